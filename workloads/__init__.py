@@ -1,0 +1,174 @@
+"""Synthetic workloads (inputs only) shared by the product path, the oracle and the bench.
+
+This module holds *inputs*: CWC model definitions (alphabet, rule strings, rates,
+initial term), run configurations (instances, horizon, sample grid, seed, histogram
+layout) and nothing of the method's arithmetic.  It is the one module both sides may
+import (task rule ③: "only the seeded input generators serve both").
+
+The paper gives no model parameters (PAPER.md L323-327 only cites [18], [20]); the
+models below are the synthetic "shaped like" workloads fixed in SURVEY.md Appendix B
+(reading R17 in DESIGN.md).  Rule order is selection order (reading R6).
+"""
+from dataclasses import dataclass, field
+from typing import Dict, List, Optional, Sequence, Tuple
+
+DEFAULT_QUANTILES = (0.05, 0.25, 0.5, 0.75, 0.95)
+
+
+@dataclass(frozen=True)
+class ModelDef:
+    """A CWC model as the C ABI receives it (cwc_model_load)."""
+
+    name: str
+    species: Tuple[str, ...]          # the alphabet of atoms, in order (species order within a region)
+    rules: Tuple[str, ...]            # "label: lhs -> rhs" strings, selection order
+    rates: Tuple[float, ...]          # one rate per rule
+    initial_term: str
+    x_cap: Optional[int] = None       # reading R9; None = model default (largest safe cap <= 2^30)
+
+
+@dataclass(frozen=True)
+class RunConfig:
+    """One BASELINE.json config, made concrete."""
+
+    cid: int
+    model: ModelDef
+    n_instances: int
+    t_end: float
+    sample_dt: float
+    seed: int
+    hist_bins: int
+    hist_width: int
+    hist_lo: int = 0
+    quantiles: Tuple[float, ...] = DEFAULT_QUANTILES
+    description: str = ""
+
+    @property
+    def n_samples(self) -> int:
+        return int(round(self.t_end / self.sample_dt)) + 1
+
+
+# --- App. B models -------------------------------------------------------------------
+
+IMM_DEATH = ModelDef(
+    name="imm_death",
+    species=("A",),
+    rules=("top: . -> A", "top: A -> ."),
+    rates=(10.0, 0.1),
+    initial_term=".",
+)
+
+# Gillespie 1977 Lotka reactions with X-bar folded into c1.
+LOTKA_VOLTERRA = ModelDef(
+    name="lotka_volterra",
+    species=("Y1", "Y2"),
+    rules=("top: Y1 -> Y1 Y1", "top: Y1 Y2 -> Y2 Y2", "top: Y2 -> ."),
+    rates=(10.0, 0.01, 10.0),
+    initial_term="1000*Y1 1000*Y2",
+    x_cap=100_000,
+)
+
+SCHLOGL = ModelDef(
+    name="schlogl",
+    species=("X",),
+    rules=("top: X X -> X X X", "top: X X X -> X X", "top: . -> X", "top: X -> ."),
+    rates=(0.03, 1e-4, 200.0, 3.5),
+    initial_term="250*X",
+)
+
+# Vilar, Kueh, Barkai, Leibler (PNAS 2002) genetic oscillator; DAp/DRp = DA'/DR'.
+CIRCADIAN = ModelDef(
+    name="circadian",
+    species=("DA", "DR", "DAp", "DRp", "MA", "MR", "A", "R", "C"),
+    rules=(
+        "top: DAp -> DA A",
+        "top: DA A -> DAp",
+        "top: DRp -> DR A",
+        "top: DR A -> DRp",
+        "top: DAp -> DAp MA",
+        "top: DA -> DA MA",
+        "top: DRp -> DRp MR",
+        "top: DR -> DR MR",
+        "top: MA -> MA A",
+        "top: MR -> MR R",
+        "top: A R -> C",
+        "top: C -> R",
+        "top: A -> .",
+        "top: R -> .",
+        "top: MA -> .",
+        "top: MR -> .",
+    ),
+    rates=(50.0, 1.0, 100.0, 1.0, 500.0, 50.0, 50.0, 0.01, 50.0, 5.0, 2.0, 1.0, 1.0, 0.2, 10.0, 0.5),
+    initial_term="DA DR",
+)
+
+# Depth-2 compartments: top ⊃ cell ⊃ nuc, receptor binding on the cell membrane,
+# transport across the nuclear membrane (SURVEY.md App. B model E).
+COMPARTMENTS = ModelDef(
+    name="compartments",
+    species=("L", "R", "RL", "S", "G", "M", "P"),
+    rules=(
+        "top: L (R $x | $X)^cell -> (RL $x | $X)^cell",
+        "top: (RL $x | $X)^cell -> L (R $x | $X)^cell",
+        "top: (RL $x | $X)^cell -> (R $x | S $X)^cell",
+        "cell: S ($y | $Y)^nuc -> ($y | S $Y)^nuc",
+        "cell: ($y | S $Y)^nuc -> S ($y | $Y)^nuc",
+        "nuc: S G -> S G M",
+        "cell: ($y | M $Y)^nuc -> M ($y | $Y)^nuc",
+        "cell: M -> M P",
+        "cell: M -> .",
+        "cell: P -> .",
+        "cell: S -> .",
+        "top: . -> L",
+        "top: L -> .",
+        "nuc: S -> .",
+    ),
+    rates=(0.01, 1.0, 0.5, 0.2, 0.1, 0.05, 1.0, 2.0, 0.2, 0.05, 0.1, 50.0, 0.1, 0.1),
+    initial_term="500*L (100*R | (. | 2*G)^nuc)^cell",
+)
+
+MODELS: Dict[str, ModelDef] = {
+    m.name: m for m in (IMM_DEATH, LOTKA_VOLTERRA, SCHLOGL, CIRCADIAN, COMPARTMENTS)
+}
+
+# --- BASELINE.json configs ------------------------------------------
+
+SEED_BASE = 0x5EED0000
+
+CONFIGS: Dict[str, RunConfig] = {
+    "imm_death": RunConfig(1, IMM_DEATH, 1_000, 100.0, 1.0, SEED_BASE + 1, 256, 1,
+                           description="immigration-death, 1,000 instances, t_end=100, dt=1"),
+    "lv": RunConfig(2, LOTKA_VOLTERRA, 100_000, 50.0, 0.1, SEED_BASE + 2, 1024, 128,
+                    description="Lotka-Volterra, 100k instances, t_end=50, dt=0.1"),
+    "schlogl": RunConfig(3, SCHLOGL, 1_000_000, 50.0, 0.1, SEED_BASE + 3, 1024, 1,
+                         description="Schlogl bistable, 1M instances, t_end=50, dt=0.1"),
+    "circadian": RunConfig(4, CIRCADIAN, 10_000_000, 48.0, 0.5, SEED_BASE + 4, 1024, 4,
+                           description="Vilar circadian oscillator, 10M instances (8 GPUs), t_end=48h, dt=0.5h"),
+    "compartments": RunConfig(5, COMPARTMENTS, 1_000_000, 100.0, 0.5, SEED_BASE + 5, 1024, 1,
+                              description="CWC cell+nucleus (depth 2, transport), 1M instances, t_end=100, dt=0.5"),
+}
+
+# --- tiny models for closed-form / CME pins -------------------------------------------------
+
+PURE_BIRTH = ModelDef("pure_birth", ("A",), ("top: . -> A",), (3.0,), ".")
+PURE_DEATH = ModelDef("pure_death", ("A",), ("top: A -> .",), (0.5,), "40*A")
+ISOMERIZATION = ModelDef("isomerization", ("A", "B"), ("top: A -> B", "top: B -> A"), (1.0, 0.5), "20*A")
+BINDING = ModelDef("binding", ("A", "B", "C"), ("top: A B -> C", "top: C -> A B"), (0.3, 1.0), "5*A 5*B")
+DIMERISATION = ModelDef("dimerisation", ("A", "B"), ("top: A A -> B", "top: B -> A A"), (0.2, 1.0), "10*A")
+DEAD = ModelDef("dead", ("A", "B"), ("top: A -> B", "top: B -> A"), (0.0, 0.0), "7*A 3*B")
+RUNAWAY = ModelDef("runaway", ("A",), ("top: A -> A A",), (1.0,), "1*A", x_cap=10)
+# transport in and out of a nucleus: S@top <-> S@nuc, a Binomial law (SURVEY.md §8(c) pins)
+TRANSPORT = ModelDef(
+    "transport", ("S",),
+    ("top: S ($y | $Y)^nuc -> ($y | S $Y)^nuc", "top: ($y | S $Y)^nuc -> S ($y | $Y)^nuc"),
+    (0.7, 0.3), "30*S (. | .)^nuc",
+)
+# two compartments with the same label (reading R15: one flat reaction per assignment)
+TWO_CELLS = ModelDef(
+    "two_cells", ("A", "B"),
+    ("top: A (. $x | $X)^cell -> (. $x | A $X)^cell", "cell: A -> B", "top: (. $x | B $X)^cell -> B (. $x | $X)^cell"),
+    (0.05, 1.0, 0.5), "20*A (. | 3*A)^cell (2*B | .)^cell",
+)
+
+TINY_MODELS = {m.name: m for m in (PURE_BIRTH, PURE_DEATH, ISOMERIZATION, BINDING, DIMERISATION,
+                                   DEAD, RUNAWAY, TRANSPORT, TWO_CELLS)}
