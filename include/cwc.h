@@ -1,0 +1,230 @@
+/*
+ * cwc.h — C ABI of the B200-native CWC ensemble stochastic simulator.
+ *
+ * The operation (PAPER.md = Aldinucci et al., ICDCS-W 2014, /root/reference/PAPER.md):
+ *   - a CWC model: an alphabet of atoms, multisets of atoms and compartments, labelled
+ *     rewrite rules local to a compartment or across compartments           P:L203-215 (§IV)
+ *   - Gillespie's stochastic simulation algorithm on CWC terms              P:L216-226 (§IV), ref [1]
+ *   - a Monte Carlo ensemble of independent instances ("trajectories")      P:L47-52 (§I)
+ *   - cuts of all trajectories at fixed simulation times, analysed on line
+ *     by statistical estimators (mean, variance; histograms/quantiles)      P:L244-252 (§IV.A)
+ *   - simulation quanta and load re-balancing on the GPU                     P:L300-317 (§IV.C)
+ * Readings of what the paper leaves open (R1-R18) are listed in DESIGN.md §3; the numeric
+ * contract (Philox stream, CWC-log, evaluation order, sampling convention) is R3-R7.
+ *
+ * Conventions
+ *   - Every function returns a cwc_status; CWC_OK == 0.  On error a thread-local message is
+ *     available from cwc_last_error() until the next cwc_* call on that thread.  No function
+ *     throws across the ABI.
+ *   - "host" pointers are ordinary CPU memory; "device" pointers are CUDA global memory of
+ *     the model's device.  All input arrays/strings are borrowed for the duration of the call
+ *     and copied; no pointer passed in is retained unless stated ("bound" buffers).
+ *   - Handles are not thread safe: one thread at a time per cwc_model_t.
+ *   - There is no CPU fallback.  Without a usable CUDA device, simulate calls return
+ *     CWC_E_CUDA; model loading, flattening and kernel code generation (NVRTC) work without one.
+ */
+#ifndef CWC_H_
+#define CWC_H_
+
+#include <stddef.h>
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+typedef int32_t cwc_status;
+#define CWC_OK 0
+#define CWC_E_INVALID 1     /* bad argument / value (null, negative, NaN, unknown atom, ...) */
+#define CWC_E_PARSE 2       /* syntax error in a term or rule */
+#define CWC_E_UNSUPPORTED 3 /* valid CWC outside the hot path: compartment creation/destruction,
+                               reaction order > 3, closed membrane patterns, moved variables */
+#define CWC_E_CUDA 4        /* CUDA / NVRTC / driver failure, or no device */
+#define CWC_E_OOM 5         /* device allocation failed */
+#define CWC_E_STATE 6       /* call out of order (e.g. stats before any simulation) */
+
+/* Per-instance flags (reading R8/R9). 0 = reached t_end. */
+#define CWC_FLAG_ABSORBED 1   /* a0 == 0: state held to t_end */
+#define CWC_FLAG_OVERFLOWED 2 /* a count exceeded x_cap: frozen, later samples missing (-1) */
+
+typedef struct cwc_model* cwc_model_t;
+
+/* ------------------------------------------------------------------------------------------
+ * Model loading — P:L203-215.
+ *   species      [n_species] atom names (the alphabet), [A-Za-z_][A-Za-z0-9_]*; their order is
+ *                the species order inside each region of the flat model.
+ *   rules        [n_rules] strings "label: lhs -> rhs"; label = "top" or a compartment label.
+ *                lhs/rhs: atoms, "n*A", "." (empty), compartments "(wrap $x | content $X)^label".
+ *                Rule order is the selection order (R6).
+ *   rates        [n_rules] mass-action rate constants, finite and >= 0.
+ *   initial_term e.g. "500*L (100*R | (. | 2*G)^nuc)^cell".
+ * The static compartment structure is flattened at load (DESIGN.md §3 "flattening"): one flat
+ * species per (region, atom), one flat reaction per (rule, context, compartment assignment).
+ * *out receives a library-owned handle (free with cwc_model_free).
+ * Errors: CWC_E_INVALID, CWC_E_PARSE, CWC_E_UNSUPPORTED.
+ * ---------------------------------------------------------------------------------------- */
+cwc_status cwc_model_load(cwc_model_t* out, int32_t n_species, const char* const* species,
+                          int32_t n_rules, const char* const* rules, const double* rates,
+                          const char* initial_term);
+
+/* Release a handle and every device buffer it owns.  NULL is a no-op. */
+void cwc_model_free(cwc_model_t m);
+
+/* Thread-local message of the last failing call ("" if none).  Valid until the next call. */
+const char* cwc_last_error(void);
+
+/* Flat view of a loaded model.  All pointers are borrowed views owned by the handle, valid
+ * until cwc_model_free (or a cwc_set_option that changes x_cap / histogram layout).
+ *   reactant_species/order: [n_reactions][4], entries beyond n_reactants[j] are 0.
+ *   delta: [n_reactions][n_species] dense net change nu_j (row-major). */
+typedef struct {
+    int32_t n_species;
+    int32_t n_reactions;
+    int32_t n_rules;
+    const char* const* species_names; /* "A", "R@cell.wrap", "S@cell/nuc", ... */
+    const int32_t* x0;
+    const double* rates;
+    const int32_t* n_reactants;
+    const int32_t* reactant_species;
+    const int32_t* reactant_order;
+    const int32_t* delta;
+    const int32_t* rule_of;           /* originating rule index of each flat reaction */
+    int64_t x_cap;                    /* current cap (R9) */
+    int64_t x_cap_max;                /* largest cap keeping every propensity count < 2^53 */
+    int32_t hist_bins;                /* B */
+    const int64_t* hist_lo;           /* [n_species] */
+    const int64_t* hist_width;        /* [n_species] */
+} cwc_model_info_t;
+cwc_status cwc_model_info(cwc_model_t m, cwc_model_info_t* out);
+
+/* ------------------------------------------------------------------------------------------
+ * Options (cwc_set_option_i64 unless noted).  Keys:
+ *   "x_cap"              1 <= v <= x_cap_max (R9).                       default x_cap_max or model's
+ *   "raw_samples"        0/1: keep the raw [T][S][count] int32 sample buffer.   default 1
+ *   "hist_bins"          B >= 1 in-range bins per (time, species).               default 256
+ *   "hist_width"         bin width >= 1 for every species;  "hist_width.<species name>" for one.
+ *   "hist_lo"            left edge of bin 1 for every species; "hist_lo.<species name>" for one.
+ *   "quantum_samples"    sample points per simulation quantum (Q/tau); 0 = auto.
+ *                        Scheduling only: results are bit-identical for every value (R12).
+ *   "block_threads"      CUDA block size (multiple of 32, <= 1024).              default 256
+ *   "blocks_per_sm"      persistent CTAs per SM; 0 = occupancy maximum.          default 0
+ *   "refill"             0/1: warp-level refill from the global work queue.      default 1
+ *   "device"             CUDA device ordinal.                                    default current
+ * cwc_set_quantiles(m, n, q): quantile levels in [0,1] (R11), default {.05,.25,.5,.75,.95}.
+ * Errors: CWC_E_INVALID (unknown key / bad value).
+ * ---------------------------------------------------------------------------------------- */
+cwc_status cwc_set_option_i64(cwc_model_t m, const char* key, int64_t value);
+cwc_status cwc_set_quantiles(cwc_model_t m, int32_t n, const double* q);
+
+/* Generate the model-specialised CUDA translation unit and compile it with NVRTC for sm_100a
+ * (cached per process and on disk by source hash).  Works without a GPU.  simulate calls it
+ * implicitly.  *source/*log (optional, may be NULL) receive borrowed views of the generated
+ * source and the NVRTC log. */
+cwc_status cwc_model_compile(cwc_model_t m, const char** source, const char** log);
+/* Compiled SASS-level facts of the last compile: registers/thread, local (spill) bytes. */
+cwc_status cwc_kernel_attributes(cwc_model_t m, int32_t* regs, int32_t* local_bytes,
+                                 int32_t* max_threads);
+
+/* ------------------------------------------------------------------------------------------
+ * Device buffers.  By default the handle allocates what it needs.  A caller that owns device
+ * memory (PyTorch) may bind its own buffers instead; they must stay valid while bound.
+ *   stats   int64[stats_len]   packed ensemble statistics (layout below)
+ *   raw     int32[raw_len]     raw samples [T][S][count] (only if raw_samples = 1)
+ *   scratch bytes              per-instance state + work queue
+ * cwc_buffer_sizes reports the sizes one cwc_simulate_range(count, t_end, dt) needs.
+ * Passing NULL pointers to cwc_bind_device_buffers unbinds (back to library allocation).
+ * ---------------------------------------------------------------------------------------- */
+cwc_status cwc_buffer_sizes(cwc_model_t m, int64_t count, double t_end, double sample_dt,
+                            size_t* stats_len, size_t* raw_len, size_t* scratch_bytes);
+cwc_status cwc_bind_device_buffers(cwc_model_t m, int64_t* stats, size_t stats_len, int32_t* raw,
+                                   size_t raw_len, void* scratch, size_t scratch_bytes);
+
+/* ------------------------------------------------------------------------------------------
+ * Simulation — the hot path.
+ * cwc_simulate_range simulates the global instances [first, first+count) of an ensemble of
+ * n_total instances, from t = 0 to t_end, sampling at t_k = fl(k*sample_dt), k = 0..K,
+ * K = llround(t_end/sample_dt) (R7, R13).  Instance i uses the Philox stream keyed by
+ * (seed, i) (R3), so any sharding of [0, n_total) gives bit-identical trajectories and
+ * statistics.  The packed stats buffer is zeroed and filled by the call.
+ * The work is enqueued on cuda_stream (a cudaStream_t; NULL = the handle's own stream) and
+ * the call returns without waiting; results are valid once the stream has drained
+ * (cwc_stats_finalize / cwc_samples / cwc_instance_records synchronise it).
+ * cwc_simulate(m, n, t_end, dt, seed) == cwc_simulate_range(m, n, 0, n, ..., NULL) followed
+ * by cwc_stats_finalize (synchronous).
+ * Errors: CWC_E_INVALID (n_total <= 0, count < 0, first+count > n_total, t_end < 0,
+ *         sample_dt <= 0, |K*dt - t_end| > 1e-9*max(1,t_end), buffers too small);
+ *         CWC_E_OOM; CWC_E_CUDA.
+ * ---------------------------------------------------------------------------------------- */
+cwc_status cwc_simulate(cwc_model_t m, int64_t n_instances, double t_end, double sample_dt,
+                        uint64_t seed);
+cwc_status cwc_simulate_range(cwc_model_t m, int64_t n_total, int64_t first, int64_t count,
+                              double t_end, double sample_dt, uint64_t seed, void* cuda_stream);
+
+/* Packed int64 statistics buffer, T = K+1 cuts, S species, B bins (all exact integers,
+ * order-independent; a sum of buffers = the buffer of the union of instance ranges):
+ *   [0, T)                       n[k]            instances present at cut k
+ *   [T, T+TS)                    sum[k][s]       sum of x
+ *   [T+TS, T+2TS)                sqlo[k][s]      sum of (x^2 mod 2^32)
+ *   [T+2TS, T+3TS)               sqhi[k][s]      sum of (x^2 >> 32)       sum x^2 = sqhi*2^32 + sqlo
+ *   [T+3TS, T+3TS+TS(B+2))       hist[k][s][b]   b=0 underflow, 1..B bins, B+1 overflow
+ *   then 8 counters:             reactions, absorbed, overflowed, finished instances, 0...
+ */
+#define CWC_CTR_REACTIONS 0
+#define CWC_CTR_ABSORBED 1
+#define CWC_CTR_OVERFLOWED 2
+#define CWC_CTR_FINISHED 3
+#define CWC_N_CTR 8
+cwc_status cwc_stats_device(cwc_model_t m, int64_t** dptr, size_t* n_int64);
+
+/* Synchronise, copy the packed stats to the host and derive mean, variance (n-1; int128
+ * numerator; NaN if n < 2) and inverted-CDF quantiles (R10, R11).  If host_stats is non-NULL
+ * the packed buffer is taken from it instead (e.g. after an NCCL all-reduce done by the
+ * caller into host memory); it must hold stats_len int64 for the last simulated geometry. */
+cwc_status cwc_stats_finalize(cwc_model_t m, const int64_t* host_stats);
+
+typedef struct {
+    int32_t T, S, B, n_q;
+    const double* times;      /* [T] t_k = fl(k*dt) */
+    const int64_t* n;         /* [T] */
+    const int64_t* sum;       /* [T*S] */
+    const double* sumsq;      /* [T*S] sum of x^2, rounded to double (exact value via sqlo/sqhi) */
+    const int64_t* sqlo;      /* [T*S] */
+    const int64_t* sqhi;      /* [T*S] */
+    const double* mean;       /* [T*S] */
+    const double* var;        /* [T*S] */
+    const int64_t* hist;      /* [T*S*(B+2)] */
+    const int64_t* hist_lo;   /* [S] */
+    const int64_t* hist_width;/* [S] */
+    const double* q;          /* [n_q] */
+    const double* quantile;   /* [T*S*n_q] (+-inf if in the under/overflow bin, NaN if n = 0) */
+    int64_t reactions, absorbed, overflowed, finished;
+    double kernel_ms;         /* device time of the last simulate kernel (CUDA events) */
+    const char* const* species_names;
+} cwc_stats_t;
+/* Borrowed views into the handle, valid until the next simulate / finalize / free. */
+cwc_status cwc_stats(cwc_model_t m, cwc_stats_t* out);
+
+/* Raw samples of local instances [first, first+count) of the last simulated range, copied to
+ * host out[T][S][count] (-1 = missing after an overflow).  CWC_E_STATE if raw_samples = 0. */
+cwc_status cwc_samples(cwc_model_t m, int64_t first, int64_t count, int32_t* out);
+
+/* Per-instance records of the last simulated range (host outputs, any may be NULL):
+ * flags (CWC_FLAG_*), reactions applied, final simulation time of the last applied reaction. */
+cwc_status cwc_instance_records(cwc_model_t m, int64_t first, int64_t count, uint8_t* flags,
+                                int64_t* reactions, double* t_last);
+
+/* ------------------------------------------------------------------------------------------
+ * Device self-tests of the hot-path primitives (the same device code the SSA kernel uses):
+ * Philox4x32-10 blocks for n (ctr, key) pairs and CWC-log for n doubles, computed on the GPU.
+ * Host arrays in, host arrays out.  ctr: [n][4], key: [n][2], out: [n][4]. */
+cwc_status cwc_selftest_philox(int64_t n, const uint32_t* ctr, const uint32_t* key, uint32_t* out);
+cwc_status cwc_selftest_log(int64_t n, const double* x, double* out);
+cwc_status cwc_selftest_u01(int64_t n, const uint32_t* words, double* out); /* words [n][2] */
+
+/* Library version string. */
+const char* cwc_version(void);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* CWC_H_ */

@@ -1,0 +1,277 @@
+"""Python API over the C ABI (include/cwc.h).  Marshalling only — every step of the hot path
+runs in the NVRTC-compiled sm_100a kernel behind ``cwc_simulate_range``.
+
+    m = Model(species, rules, rates, initial_term, x_cap=..., hist_bins=..., hist_width=...)
+    res = m.simulate(n_instances, t_end, sample_dt, seed)      # synchronous, host results
+    res.mean[k, s], res.var[k, s], res.quantile[k, s, q], res.hist[k, s, b]
+
+PyTorch only provides device memory and streams: ``DeviceBuffers`` allocates the stats / raw /
+scratch buffers as torch tensors and binds them, and ``simulate_range`` enqueues on a torch
+stream so the caller can time it with CUDA events and all-reduce the stats with NCCL.
+"""
+from __future__ import annotations
+
+import ctypes
+from dataclasses import dataclass
+from typing import List, Optional, Sequence
+
+import numpy as np
+
+from . import _lib
+from ._lib import CWCError, check, lib  # noqa: F401
+
+
+def _ptr(a: np.ndarray):
+    return ctypes.c_void_p(a.ctypes.data)
+
+
+@dataclass
+class EnsembleResult:
+    """Finalised ensemble statistics of one simulation (cwc_stats_t as numpy arrays)."""
+
+    times: np.ndarray       # [T]
+    n: np.ndarray           # [T] int64
+    sum: np.ndarray         # [T,S] int64
+    sqlo: np.ndarray        # [T,S] int64
+    sqhi: np.ndarray        # [T,S] int64
+    sumsq: np.ndarray       # [T,S] float64 (rounded)
+    mean: np.ndarray        # [T,S]
+    var: np.ndarray         # [T,S]
+    hist: np.ndarray        # [T,S,B+2] int64
+    hist_lo: np.ndarray     # [S]
+    hist_width: np.ndarray  # [S]
+    q: np.ndarray           # [Q]
+    quantile: np.ndarray    # [T,S,Q]
+    reactions: int
+    absorbed: int
+    overflowed: int
+    finished: int
+    kernel_ms: float
+    species: List[str]
+
+    def sumsq_exact(self) -> np.ndarray:
+        out = np.empty(self.sqlo.shape, dtype=object)
+        for idx in np.ndindex(self.sqlo.shape):
+            out[idx] = (int(self.sqhi[idx]) << 32) + int(self.sqlo[idx])
+        return out
+
+
+class Model:
+    """A loaded CWC model (cwc_model_load) with its options."""
+
+    def __init__(self, species: Sequence[str], rules: Sequence[str], rates: Sequence[float], initial_term: str,
+                 *, x_cap: Optional[int] = None, hist_bins: Optional[int] = None, hist_width=None, hist_lo=None,
+                 quantiles: Optional[Sequence[float]] = None, raw_samples: bool = True,
+                 quantum_samples: int = 0, block_threads: Optional[int] = None, refill: bool = True,
+                 device: Optional[int] = None):
+        sp = (ctypes.c_char_p * len(species))(*[s.encode() for s in species])
+        rl = (ctypes.c_char_p * max(len(rules), 1))(*[r.encode() for r in rules])
+        rt = (ctypes.c_double * max(len(rates), 1))(*[float(k) for k in rates])
+        h = ctypes.c_void_p()
+        check(lib.cwc_model_load(ctypes.byref(h), len(species), sp, len(rules), rl, rt, initial_term.encode()))
+        self._h = h
+        self._info_cache = None
+        if x_cap is not None:
+            self.set_option("x_cap", int(x_cap))
+        if hist_bins is not None:
+            self.set_option("hist_bins", int(hist_bins))
+        for key, val in (("hist_width", hist_width), ("hist_lo", hist_lo)):
+            if val is None:
+                continue
+            if isinstance(val, dict):
+                for name, v in val.items():
+                    self.set_option(f"{key}.{name}", int(v))
+            else:
+                self.set_option(key, int(val))
+        if quantiles is not None:
+            self.set_quantiles(quantiles)
+        self.set_option("raw_samples", 1 if raw_samples else 0)
+        self.set_option("quantum_samples", int(quantum_samples))
+        if block_threads is not None:
+            self.set_option("block_threads", int(block_threads))
+        self.set_option("refill", 1 if refill else 0)
+        if device is not None:
+            self.set_option("device", int(device))
+
+    @classmethod
+    def from_def(cls, mdef, **kw) -> "Model":
+        """Load a workloads.ModelDef-like object (species, rules, rates, initial_term, x_cap)."""
+        if getattr(mdef, "x_cap", None) is not None and "x_cap" not in kw:
+            kw["x_cap"] = mdef.x_cap
+        return cls(mdef.species, mdef.rules, mdef.rates, mdef.initial_term, **kw)
+
+    def close(self):
+        if getattr(self, "_h", None):
+            lib.cwc_model_free(self._h)
+            self._h = None
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+    @property
+    def handle(self):
+        return self._h
+
+    # ---------------------------------------------------------------- options / info
+    def set_option(self, key: str, value: int) -> None:
+        check(lib.cwc_set_option_i64(self._h, key.encode(), int(value)))
+        self._info_cache = None
+
+    def set_quantiles(self, qs: Sequence[float]) -> None:
+        arr = (ctypes.c_double * max(len(qs), 1))(*[float(q) for q in qs])
+        check(lib.cwc_set_quantiles(self._h, len(qs), arr))
+
+    def info(self) -> dict:
+        if self._info_cache is None:
+            mi = _lib.ModelInfo()
+            check(lib.cwc_model_info(self._h, ctypes.byref(mi)))
+            S, M = mi.n_species, mi.n_reactions
+            nre = [mi.n_reactants[j] for j in range(M)]
+            self._info_cache = dict(
+                names=[mi.species_names[s].decode() for s in range(S)],
+                x0=[mi.x0[s] for s in range(S)],
+                rates=[mi.rates[j] for j in range(M)],
+                reactants=[[(mi.reactant_species[j * 4 + e], mi.reactant_order[j * 4 + e]) for e in range(nre[j])]
+                           for j in range(M)],
+                delta=[[mi.delta[j * S + s] for s in range(S)] for j in range(M)],
+                rule_of=[mi.rule_of[j] for j in range(M)],
+                x_cap=mi.x_cap, x_cap_max=mi.x_cap_max, n_rules=mi.n_rules, hist_bins=mi.hist_bins,
+                hist_lo=[mi.hist_lo[s] for s in range(S)], hist_width=[mi.hist_width[s] for s in range(S)],
+            )
+        return self._info_cache
+
+    @property
+    def n_species(self) -> int:
+        return len(self.info()["names"])
+
+    def compile(self):
+        """NVRTC-compile the model's kernel for sm_100a (no GPU needed); returns (source, log)."""
+        src, log = ctypes.c_char_p(), ctypes.c_char_p()
+        check(lib.cwc_model_compile(self._h, ctypes.byref(src), ctypes.byref(log)))
+        return src.value.decode(), log.value.decode()
+
+    def kernel_attributes(self) -> dict:
+        r, l, t = ctypes.c_int32(), ctypes.c_int32(), ctypes.c_int32()
+        check(lib.cwc_kernel_attributes(self._h, ctypes.byref(r), ctypes.byref(l), ctypes.byref(t)))
+        return dict(registers=r.value, local_bytes=l.value, max_threads=t.value)
+
+    def buffer_sizes(self, count: int, t_end: float, dt: float):
+        a, b, c = ctypes.c_size_t(), ctypes.c_size_t(), ctypes.c_size_t()
+        check(lib.cwc_buffer_sizes(self._h, int(count), float(t_end), float(dt), ctypes.byref(a), ctypes.byref(b),
+                                   ctypes.byref(c)))
+        return a.value, b.value, c.value
+
+    # ---------------------------------------------------------------- simulation
+    def simulate(self, n_instances: int, t_end: float, sample_dt: float, seed: int) -> EnsembleResult:
+        """The public end-to-end call: simulate n instances, return host statistics."""
+        check(lib.cwc_simulate(self._h, int(n_instances), float(t_end), float(sample_dt), int(seed)))
+        return self.stats()
+
+    def simulate_range(self, n_total: int, first: int, count: int, t_end: float, sample_dt: float, seed: int,
+                       stream=None) -> None:
+        """Enqueue instances [first, first+count) on ``stream`` (a torch.cuda.Stream, a raw
+        cudaStream_t int, or None for the handle's own stream).  Asynchronous."""
+        if stream is not None and hasattr(stream, "cuda_stream"):
+            stream = stream.cuda_stream
+        check(lib.cwc_simulate_range(self._h, int(n_total), int(first), int(count), float(t_end),
+                                     float(sample_dt), int(seed), ctypes.c_void_p(stream or 0)))
+
+    def finalize(self, host_stats: Optional[np.ndarray] = None) -> EnsembleResult:
+        if host_stats is not None:
+            host_stats = np.ascontiguousarray(host_stats, dtype=np.int64)
+            check(lib.cwc_stats_finalize(self._h, _ptr(host_stats)))
+        else:
+            check(lib.cwc_stats_finalize(self._h, None))
+        return self.stats()
+
+    def stats(self) -> EnsembleResult:
+        st = _lib.Stats()
+        check(lib.cwc_stats(self._h, ctypes.byref(st)))
+        T, S, B, Q = st.T, st.S, st.B, st.n_q
+
+        def arr(p, n, dt, shape):
+            return np.ctypeslib.as_array(p, shape=(n,)).astype(dt, copy=True).reshape(shape)
+
+        return EnsembleResult(
+            times=arr(st.times, T, np.float64, (T,)), n=arr(st.n, T, np.int64, (T,)),
+            sum=arr(st.sum, T * S, np.int64, (T, S)), sqlo=arr(st.sqlo, T * S, np.int64, (T, S)),
+            sqhi=arr(st.sqhi, T * S, np.int64, (T, S)), sumsq=arr(st.sumsq, T * S, np.float64, (T, S)),
+            mean=arr(st.mean, T * S, np.float64, (T, S)), var=arr(st.var, T * S, np.float64, (T, S)),
+            hist=arr(st.hist, T * S * (B + 2), np.int64, (T, S, B + 2)),
+            hist_lo=arr(st.hist_lo, S, np.int64, (S,)), hist_width=arr(st.hist_width, S, np.int64, (S,)),
+            q=arr(st.q, Q, np.float64, (Q,)) if Q else np.zeros(0),
+            quantile=arr(st.quantile, T * S * Q, np.float64, (T, S, Q)) if Q else np.zeros((T, S, 0)),
+            reactions=st.reactions, absorbed=st.absorbed, overflowed=st.overflowed, finished=st.finished,
+            kernel_ms=st.kernel_ms, species=[st.species_names[s].decode() for s in range(S)],
+        )
+
+    def stats_device(self):
+        p, n = ctypes.c_void_p(), ctypes.c_size_t()
+        check(lib.cwc_stats_device(self._h, ctypes.byref(p), ctypes.byref(n)))
+        return p.value, n.value
+
+    def samples(self, first: int, count: int) -> np.ndarray:
+        info = self.info()
+        n_t = self.stats_T()
+        out = np.empty((n_t, len(info["names"]), count), dtype=np.int32)
+        check(lib.cwc_samples(self._h, int(first), int(count), _ptr(out)))
+        return out
+
+    def stats_T(self) -> int:
+        st = _lib.Stats()
+        if lib.cwc_stats(self._h, ctypes.byref(st)) == 0:
+            return st.T
+        raise CWCError(6, "finalize before reading samples")
+
+    def records(self, first: int, count: int):
+        flags = np.empty(count, dtype=np.uint8)
+        reactions = np.empty(count, dtype=np.int64)
+        t_last = np.empty(count, dtype=np.float64)
+        check(lib.cwc_instance_records(self._h, int(first), int(count), _ptr(flags), _ptr(reactions), _ptr(t_last)))
+        return flags, reactions, t_last
+
+
+class DeviceBuffers:
+    """Torch-owned device buffers bound to a model for one (count, t_end, dt) geometry."""
+
+    def __init__(self, model: Model, count: int, t_end: float, sample_dt: float, device=None):
+        import torch
+        n_stats, n_raw, n_scratch = model.buffer_sizes(count, t_end, sample_dt)
+        dev = torch.device("cuda", torch.cuda.current_device()) if device is None else torch.device(device)
+        self.stats = torch.empty(n_stats, dtype=torch.int64, device=dev)
+        self.raw = torch.empty(max(n_raw, 1), dtype=torch.int32, device=dev) if n_raw else None
+        self.scratch = torch.empty(n_scratch, dtype=torch.uint8, device=dev)
+        self.model = model
+        model.set_option("device", dev.index)
+        check(lib.cwc_bind_device_buffers(
+            model.handle, ctypes.c_void_p(self.stats.data_ptr()), n_stats,
+            ctypes.c_void_p(self.raw.data_ptr() if self.raw is not None else 0), n_raw,
+            ctypes.c_void_p(self.scratch.data_ptr()), n_scratch))
+
+    def unbind(self):
+        check(lib.cwc_bind_device_buffers(self.model.handle, None, 0, None, 0, None, 0))
+
+
+def selftest_philox(ctr: np.ndarray, key: np.ndarray) -> np.ndarray:
+    ctr = np.ascontiguousarray(ctr, dtype=np.uint32).reshape(-1, 4)
+    key = np.ascontiguousarray(key, dtype=np.uint32).reshape(-1, 2)
+    out = np.empty_like(ctr)
+    check(lib.cwc_selftest_philox(len(ctr), _ptr(ctr), _ptr(key), _ptr(out)))
+    return out
+
+
+def selftest_log(x: np.ndarray) -> np.ndarray:
+    x = np.ascontiguousarray(x, dtype=np.float64)
+    out = np.empty_like(x)
+    check(lib.cwc_selftest_log(len(x), _ptr(x), _ptr(out)))
+    return out
+
+
+def selftest_u01(words: np.ndarray) -> np.ndarray:
+    w = np.ascontiguousarray(words, dtype=np.uint32).reshape(-1, 2)
+    out = np.empty(len(w), dtype=np.float64)
+    check(lib.cwc_selftest_u01(len(w), _ptr(w), _ptr(out)))
+    return out

@@ -1,0 +1,333 @@
+// abi.cpp — the extern "C" boundary declared in include/cwc.h.  Argument checking, option
+// handling and exception -> status translation; the work is in compiler.cpp / runtime.cpp.
+#include <cmath>
+#include <cstring>
+#include <new>
+#include <string>
+
+#include "cwc.h"
+#include "runtime.hpp"
+
+namespace {
+
+thread_local std::string g_err;
+
+template <class F>
+cwc_status guard(F&& f) {
+    g_err.clear();
+    try {
+        f();
+        return CWC_OK;
+    } catch (const cwc::Error& e) {
+        g_err = e.what();
+        return e.code;
+    } catch (const std::bad_alloc&) {
+        g_err = "host out of memory";
+        return CWC_E_OOM;
+    } catch (const std::exception& e) {
+        g_err = e.what();
+        return CWC_E_INVALID;
+    } catch (...) {
+        g_err = "unknown error";
+        return CWC_E_INVALID;
+    }
+}
+
+[[noreturn]] void fail(int32_t code, const std::string& msg) { throw cwc::Error(code, msg); }
+
+void need(bool c, const char* msg) {
+    if (!c) fail(CWC_E_INVALID, msg);
+}
+
+void refresh_info(cwc_model* m) {
+    const cwc::FlatModel& fm = m->fm;
+    const int S = fm.S(), M = fm.M();
+    m->name_ptrs.clear();
+    for (auto& n : fm.names) m->name_ptrs.push_back(n.c_str());
+    m->info_nreact.assign(M, 0);
+    m->info_rspecies.assign((size_t)M * 4, 0);
+    m->info_rorder.assign((size_t)M * 4, 0);
+    m->info_delta.assign((size_t)M * S, 0);
+    for (int j = 0; j < M; ++j) {
+        m->info_nreact[j] = (int32_t)fm.reactants[j].size();
+        for (size_t e = 0; e < fm.reactants[j].size(); ++e) {
+            m->info_rspecies[j * 4 + e] = fm.reactants[j][e].species;
+            m->info_rorder[j * 4 + e] = fm.reactants[j][e].order;
+        }
+        for (int s = 0; s < S; ++s) m->info_delta[(size_t)j * S + s] = fm.delta[j][s];
+    }
+}
+
+int species_index(const cwc_model* m, const std::string& name) {
+    for (int s = 0; s < m->fm.S(); ++s)
+        if (m->fm.names[s] == name) return s;
+    fail(CWC_E_INVALID, "unknown species '" + name + "'");
+}
+
+}  // namespace
+
+extern "C" {
+
+const char* cwc_version(void) { return "cwc-b200 0.1 (sm_100a, NVRTC-specialised SSA)"; }
+
+const char* cwc_last_error(void) { return g_err.c_str(); }
+
+cwc_status cwc_model_load(cwc_model_t* out, int32_t n_species, const char* const* species, int32_t n_rules,
+                          const char* const* rules, const double* rates, const char* initial_term) {
+    return guard([&] {
+        need(out != nullptr, "out is NULL");
+        *out = nullptr;
+        need(n_species > 0 && species != nullptr, "need at least one species");
+        need(n_rules >= 0 && (n_rules == 0 || (rules != nullptr && rates != nullptr)), "bad rule arrays");
+        need(initial_term != nullptr, "initial_term is NULL");
+        std::vector<std::string> alpha, rs;
+        std::vector<double> ks;
+        for (int i = 0; i < n_species; ++i) {
+            need(species[i] != nullptr, "NULL species name");
+            alpha.emplace_back(species[i]);
+        }
+        for (int i = 0; i < n_rules; ++i) {
+            need(rules[i] != nullptr, "NULL rule");
+            rs.emplace_back(rules[i]);
+            ks.push_back(rates[i]);
+        }
+        cwc::FlatModel fm = cwc::compile_model(alpha, rs, ks, initial_term);
+        cwc_model* m = new cwc_model();
+        m->fm = std::move(fm);
+        m->x_cap = m->fm.x_cap_max;
+        for (int32_t v : m->fm.x0)
+            if (v > m->x_cap) {
+                delete m;
+                fail(CWC_E_INVALID, "initial count above the largest exact cap");
+            }
+        m->hist_lo.assign(m->fm.S(), 0);
+        m->hist_width.assign(m->fm.S(), 1);
+        refresh_info(m);
+        *out = m;
+    });
+}
+
+void cwc_model_free(cwc_model_t m) {
+    try {
+        delete m;
+    } catch (...) {
+    }
+}
+
+cwc_status cwc_model_info(cwc_model_t m, cwc_model_info_t* out) {
+    return guard([&] {
+        need(m && out, "NULL argument");
+        out->n_species = m->fm.S();
+        out->n_reactions = m->fm.M();
+        out->n_rules = m->fm.n_rules;
+        out->species_names = m->name_ptrs.data();
+        out->x0 = m->fm.x0.data();
+        out->rates = m->fm.rates.data();
+        out->n_reactants = m->info_nreact.data();
+        out->reactant_species = m->info_rspecies.data();
+        out->reactant_order = m->info_rorder.data();
+        out->delta = m->info_delta.data();
+        out->rule_of = m->fm.rule_of.data();
+        out->x_cap = m->x_cap;
+        out->x_cap_max = m->fm.x_cap_max;
+        out->hist_bins = m->hist_bins;
+        out->hist_lo = m->hist_lo.data();
+        out->hist_width = m->hist_width.data();
+    });
+}
+
+cwc_status cwc_set_option_i64(cwc_model_t m, const char* key, int64_t v) {
+    return guard([&] {
+        need(m && key, "NULL argument");
+        std::string k(key);
+        if (k == "x_cap") {
+            need(v >= 1 && v <= m->fm.x_cap_max, "x_cap outside [1, x_cap_max]");
+            for (int32_t x : m->fm.x0) need(x <= v, "x_cap below an initial count");
+            m->x_cap = v;
+        } else if (k == "raw_samples") {
+            need(v == 0 || v == 1, "raw_samples is 0 or 1");
+            m->raw_samples = (int)v;
+        } else if (k == "hist_bins") {
+            need(v >= 1 && v <= (1 << 20), "hist_bins outside [1, 2^20]");
+            m->hist_bins = (int)v;
+        } else if (k == "hist_width") {
+            need(v >= 1 && v <= (int64_t)1 << 40, "hist_width must be >= 1");
+            m->hist_width.assign(m->fm.S(), v);
+        } else if (k.rfind("hist_width.", 0) == 0) {
+            need(v >= 1 && v <= (int64_t)1 << 40, "hist_width must be >= 1");
+            m->hist_width[species_index(m, k.substr(11))] = v;
+        } else if (k == "hist_lo") {
+            need(std::llabs(v) <= (int64_t)1 << 40, "hist_lo out of range");
+            m->hist_lo.assign(m->fm.S(), v);
+        } else if (k.rfind("hist_lo.", 0) == 0) {
+            need(std::llabs(v) <= (int64_t)1 << 40, "hist_lo out of range");
+            m->hist_lo[species_index(m, k.substr(8))] = v;
+        } else if (k == "quantum_samples") {
+            need(v >= 0, "quantum_samples must be >= 0");
+            m->quantum_samples = v;
+        } else if (k == "block_threads") {
+            need(v >= 32 && v <= 1024 && v % 32 == 0, "block_threads: multiple of 32 in [32, 1024]");
+            m->block_threads = (int)v;
+        } else if (k == "blocks_per_sm") {
+            need(v >= 0 && v <= 64, "blocks_per_sm in [0, 64]");
+            m->blocks_per_sm = (int)v;
+        } else if (k == "refill") {
+            need(v == 0 || v == 1, "refill is 0 or 1");
+            m->refill = (int)v;
+        } else if (k == "device") {
+            need(v >= -1 && v < 1024, "bad device ordinal");
+            m->device = (int)v;
+        } else {
+            fail(CWC_E_INVALID, "unknown option '" + k + "'");
+        }
+    });
+}
+
+cwc_status cwc_set_quantiles(cwc_model_t m, int32_t n, const double* q) {
+    return guard([&] {
+        need(m && n >= 0 && (n == 0 || q), "bad quantile arguments");
+        std::vector<double> v(q, q + n);
+        for (double x : v) need(x >= 0 && x <= 1, "quantile levels must be in [0, 1]");
+        m->quantiles = v;
+    });
+}
+
+cwc_status cwc_model_compile(cwc_model_t m, const char** source, const char** log) {
+    return guard([&] {
+        need(m != nullptr, "NULL model");
+        cwc::compile(m);
+        if (source) *source = m->source.c_str();
+        if (log) *log = m->nvrtc_log.c_str();
+    });
+}
+
+cwc_status cwc_kernel_attributes(cwc_model_t m, int32_t* regs, int32_t* local_bytes, int32_t* max_threads) {
+    return guard([&] {
+        need(m != nullptr, "NULL model");
+        if (m->cubin.empty()) fail(CWC_E_STATE, "kernel not compiled");
+        if (regs) *regs = m->regs;
+        if (local_bytes) *local_bytes = m->local_bytes;
+        if (max_threads) *max_threads = m->max_threads;
+    });
+}
+
+cwc_status cwc_buffer_sizes(cwc_model_t m, int64_t count, double t_end, double dt, size_t* stats, size_t* raw,
+                            size_t* scratch) {
+    return guard([&] {
+        need(m != nullptr && count >= 0, "bad arguments");
+        int64_t K = cwc::grid_K(t_end, dt);
+        cwc::buffer_sizes(m, count, K, stats, raw, scratch);
+    });
+}
+
+cwc_status cwc_bind_device_buffers(cwc_model_t m, int64_t* stats, size_t stats_len, int32_t* raw, size_t raw_len,
+                                   void* scratch, size_t scratch_bytes) {
+    return guard([&] {
+        need(m != nullptr, "NULL model");
+        cwc::bind_buffers(m, stats, stats_len, raw, raw_len, scratch, scratch_bytes);
+    });
+}
+
+cwc_status cwc_simulate_range(cwc_model_t m, int64_t n_total, int64_t first, int64_t count, double t_end,
+                              double dt, uint64_t seed, void* stream) {
+    return guard([&] {
+        need(m != nullptr, "NULL model");
+        cwc::simulate_range(m, n_total, first, count, t_end, dt, seed, (cudaStream_t)stream);
+    });
+}
+
+cwc_status cwc_simulate(cwc_model_t m, int64_t n, double t_end, double dt, uint64_t seed) {
+    return guard([&] {
+        need(m != nullptr, "NULL model");
+        cwc::simulate_range(m, n, 0, n, t_end, dt, seed, nullptr);
+        cwc::finalize(m, nullptr);
+    });
+}
+
+cwc_status cwc_stats_device(cwc_model_t m, int64_t** dptr, size_t* n) {
+    return guard([&] {
+        need(m && dptr && n, "NULL argument");
+        if (!m->simulated) fail(CWC_E_STATE, "no simulation yet");
+        *dptr = m->d_stats;
+        *n = m->last_stats_len;
+    });
+}
+
+cwc_status cwc_stats_finalize(cwc_model_t m, const int64_t* host_stats) {
+    return guard([&] {
+        need(m != nullptr, "NULL model");
+        cwc::finalize(m, host_stats);
+    });
+}
+
+cwc_status cwc_stats(cwc_model_t m, cwc_stats_t* out) {
+    return guard([&] {
+        need(m && out, "NULL argument");
+        if (!m->finalized) fail(CWC_E_STATE, "call cwc_stats_finalize after simulating");
+        const int64_t T = m->K + 1;
+        const int S = m->fm.S();
+        std::memset(out, 0, sizeof *out);
+        out->T = (int32_t)T;
+        out->S = S;
+        out->B = m->hist_bins;
+        out->n_q = (int32_t)m->quantiles.size();
+        out->times = m->times.data();
+        out->n = m->h_n.data();
+        out->sum = m->h_sum.data();
+        out->sumsq = m->sumsq_d.data();
+        out->sqlo = m->h_sqlo.data();
+        out->sqhi = m->h_sqhi.data();
+        out->mean = m->mean.data();
+        out->var = m->var.data();
+        out->hist = m->h_hist.data();
+        out->hist_lo = m->hist_lo.data();
+        out->hist_width = m->hist_width.data();
+        out->q = m->quantiles.data();
+        out->quantile = m->quant.data();
+        const int64_t* ctr = m->h_stats.data() + T * (1 + 3 * (int64_t)S + (int64_t)S * (m->hist_bins + 2));
+        out->reactions = ctr[CWC_CTR_REACTIONS];
+        out->absorbed = ctr[CWC_CTR_ABSORBED];
+        out->overflowed = ctr[CWC_CTR_OVERFLOWED];
+        out->finished = ctr[CWC_CTR_FINISHED];
+        out->kernel_ms = m->kernel_ms;
+        out->species_names = m->name_ptrs.data();
+    });
+}
+
+cwc_status cwc_samples(cwc_model_t m, int64_t first, int64_t count, int32_t* out) {
+    return guard([&] {
+        need(m != nullptr, "NULL model");
+        cwc::copy_samples(m, first, count, out);
+    });
+}
+
+cwc_status cwc_instance_records(cwc_model_t m, int64_t first, int64_t count, uint8_t* flags, int64_t* reactions,
+                                double* t_last) {
+    return guard([&] {
+        need(m != nullptr, "NULL model");
+        cwc::copy_records(m, first, count, flags, reactions, t_last);
+    });
+}
+
+cwc_status cwc_selftest_philox(int64_t n, const uint32_t* ctr, const uint32_t* key, uint32_t* out) {
+    return guard([&] {
+        need(n >= 0 && (n == 0 || (ctr && key && out)), "bad arguments");
+        cwc::selftest_philox(n, ctr, key, out);
+    });
+}
+
+cwc_status cwc_selftest_log(int64_t n, const double* x, double* out) {
+    return guard([&] {
+        need(n >= 0 && (n == 0 || (x && out)), "bad arguments");
+        cwc::selftest_log(n, x, out);
+    });
+}
+
+cwc_status cwc_selftest_u01(int64_t n, const uint32_t* w, double* out) {
+    return guard([&] {
+        need(n >= 0 && (n == 0 || (w && out)), "bad arguments");
+        cwc::selftest_u01(n, w, out);
+    });
+}
+
+}  // extern "C"

@@ -1,0 +1,115 @@
+// codegen.cpp — emit the model section of the SSA kernel translation unit.
+//
+// The flat network from the rule compiler becomes straight-line CUDA: species counts are an
+// int array indexed only by compile-time constants (registers), rate constants are exact hex
+// literals, propensities are the product of per-species binomial factors (R1) multiplied by
+// k_j and summed left to right with explicitly rounded operations (R5), and the rewrite
+// x += nu_{j*} is a predicated select chain (no divergent branch on the selected rule).
+#include "codegen.hpp"
+
+#include <cstdio>
+#include <sstream>
+
+namespace cwc {
+namespace {
+
+std::string hexd(double v) {
+    char buf[64];
+    std::snprintf(buf, sizeof buf, "%a", v);
+    return buf;
+}
+
+}  // namespace
+
+std::string generate_model_section(const FlatModel& fm, const KernelConfig& cfg) {
+    const int S = fm.S(), M = fm.M();
+    std::ostringstream o;
+    o << "// ---- generated model section: " << S << " species, " << M << " flat reactions\n";
+    o << "#define CWC_S " << S << "\n#define CWC_M " << (M > 0 ? M : 1) << "\n#define CWC_B " << cfg.hist_bins
+      << "\n#define CWC_BLOCK " << cfg.block_threads << "\n";
+    o << "#define CWC_X_CAP " << cfg.x_cap << "\n\n";
+    for (int s = 0; s < S; ++s) o << "// species " << s << ": " << fm.names[s] << "\n";
+
+    // x = x0
+    o << "__device__ __forceinline__ void cwc_init(int (&x)[CWC_S]) {\n";
+    for (int s = 0; s < S; ++s) o << "    x[" << s << "] = " << fm.x0[s] << ";\n";
+    o << "}\n\n";
+
+    // propensities: emitted twice, as the running sums (hot) and as "last a_j > 0" (the rare
+    // rounding-hole fallback of R6) so only cum[] is live across the step.
+    for (int variant = 0; variant < 2; ++variant) {
+    if (variant == 0)
+        o << "__device__ __forceinline__ double cwc_propensities(const int (&x)[CWC_S], double (&cum)[CWC_M]) {\n"
+             "    double a[CWC_M];\n";
+    else
+        o << "__device__ __forceinline__ int cwc_last_positive(const int (&x)[CWC_S]) {\n    double a[CWC_M];\n";
+    // per-(species, order) binomial factors, shared between reactions
+    std::vector<std::vector<bool>> need(S, std::vector<bool>(4, false));
+    for (int j = 0; j < M; ++j)
+        for (const Reactant& r : fm.reactants[j]) need[r.species][r.order] = true;
+    for (int s = 0; s < S; ++s) {
+        if (need[s][1] || need[s][2]) o << "    const double f" << s << "_1 = (double)x[" << s << "];\n";
+        if (need[s][2])
+            o << "    const double f" << s << "_2 = __dmul_rn(__dmul_rn(f" << s << "_1, (double)(x[" << s << "] > 0 ? x["
+              << s << "] - 1 : 0)), 0.5);\n";
+        if (need[s][3])
+            o << "    const double f" << s << "_3 = (double)(((long long)x[" << s << "] * (long long)(x[" << s
+              << "] - 1) / 2) * (long long)(x[" << s << "] - 2) / 3);\n";
+    }
+    if (M == 0) o << "    a[0] = 0.0;\n";
+    for (int j = 0; j < M; ++j) {
+        std::string h;
+        for (const Reactant& r : fm.reactants[j]) {
+            std::string f = "f" + std::to_string(r.species) + "_" + std::to_string(r.order);
+            h = h.empty() ? f : "__dmul_rn(" + h + ", " + f + ")";
+        }
+        o << "    a[" << j << "] = " << (h.empty() ? hexd(fm.rates[j]) : "__dmul_rn(" + hexd(fm.rates[j]) + ", " + h + ")")
+          << ";  // rule " << fm.rule_of[j] << "\n";
+    }
+    if (variant == 0) {
+        o << "    cum[0] = a[0];\n";
+        for (int j = 1; j < M; ++j) o << "    cum[" << j << "] = __dadd_rn(cum[" << j - 1 << "], a[" << j << "]);\n";
+        o << "    return cum[CWC_M - 1];\n}\n\n";
+    } else {
+        o << "    int j = 0;\n#pragma unroll\n    for (int i = 0; i < CWC_M; ++i) if (a[i] > 0.0) j = i;\n";
+        o << "    return j;\n}\n\n";
+    }
+    }
+
+    // selection: j* = min{j : cum_j > target} = #{j : cum_j <= target}; rounding hole -> last a_j > 0
+    o << "__device__ __forceinline__ int cwc_select(const int (&x)[CWC_S], const double (&cum)[CWC_M], double target) {\n";
+    o << "    int j = 0;\n";
+    o << "#pragma unroll\n    for (int i = 0; i < CWC_M; ++i) j += (cum[i] <= target) ? 1 : 0;\n";
+    o << "    if (j >= CWC_M) j = cwc_last_positive(x);\n";
+    o << "    return j;\n}\n\n";
+
+    // rewrite + overflow check on the species some rule increases
+    o << "__device__ __forceinline__ bool cwc_apply(int j, int (&x)[CWC_S]) {\n";
+    std::vector<bool> inc(S, false);
+    for (int s = 0; s < S; ++s) {
+        std::string chain = "0";
+        for (int j = M - 1; j >= 0; --j) {
+            int d = fm.delta[j][s];
+            if (!d) continue;
+            if (d > 0) inc[s] = true;
+            chain = "(j == " + std::to_string(j) + " ? " + std::to_string(d) + " : " + chain + ")";
+        }
+        if (chain != "0") o << "    x[" << s << "] += " << chain << ";\n";
+    }
+    o << "    bool over = false;\n";
+    for (int s = 0; s < S; ++s)
+        if (inc[s]) o << "    over |= x[" << s << "] > CWC_X_CAP;\n";
+    o << "    return over;\n}\n\n";
+
+    // histogram bins: 0 underflow, 1..B, B+1 overflow (R11)
+    o << "__device__ __forceinline__ int cwc_bin(int s, int v) {\n    long long lo = 0, w = 1;\n    switch (s) {\n";
+    for (int s = 0; s < S; ++s)
+        o << "        case " << s << ": lo = " << cfg.hist_lo[s] << "LL; w = " << cfg.hist_width[s] << "LL; break;\n";
+    o << "        default: break;\n    }\n";
+    o << "    const long long d = (long long)v - lo;\n";
+    o << "    if (d < 0) return 0;\n    const long long b = d / w;\n    return b >= CWC_B ? CWC_B + 1 : (int)b + 1;\n}\n";
+    o << "// ---- end of generated model section\n\n";
+    return o.str();
+}
+
+}  // namespace cwc

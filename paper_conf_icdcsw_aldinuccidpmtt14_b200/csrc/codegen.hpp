@@ -1,0 +1,24 @@
+// codegen.hpp — model-specialised CUDA source generation.
+#pragma once
+
+#include <string>
+#include <vector>
+
+#include "compiler.hpp"
+
+namespace cwc {
+
+struct KernelConfig {
+    int block_threads = 256;
+    int hist_bins = 256;
+    int64_t x_cap = 0;
+    std::vector<int64_t> hist_lo, hist_width;  // [S]
+};
+
+// The model section (macros + inline device functions) consumed by device/cwc_ssa.cuh.
+std::string generate_model_section(const FlatModel& fm, const KernelConfig& cfg);
+
+// Full NVRTC translation unit: cwc_params.h + cwc_rng.cuh + model section + cwc_ssa.cuh.
+std::string generate_kernel_source(const FlatModel& fm, const KernelConfig& cfg);
+
+}  // namespace cwc

@@ -1,0 +1,53 @@
+// Rule compiler: CWC terms + rewrite rules -> flat mass-action network.
+//
+// PAPER.md P:L203-215 (§IV): CWC terms are multisets of atoms and compartments; a compartment
+// has a membrane (wrap) multiset, a content term and a label; rules rewrite inside a compartment
+// or across nested compartments.  The paper's simulator matches rule patterns against dynamic
+// term trees at every step.  For static compartment structure (no creation or
+// destruction, R15/R16) every match site is fixed, so this compiler does the tree matching ONCE
+// at load and emits one flat reaction per (rule, context, compartment assignment); the GPU then
+// never touches a tree.  DESIGN.md §3 "flattening" is the normative statement.
+#pragma once
+
+#include <cstdint>
+#include <stdexcept>
+#include <string>
+#include <vector>
+
+namespace cwc {
+
+struct Error : std::runtime_error {
+    int32_t code;  // CWC_E_*
+    Error(int32_t c, const std::string& m) : std::runtime_error(m), code(c) {}
+};
+
+struct Reactant {
+    int32_t species;
+    int32_t order;
+    bool operator==(const Reactant& o) const { return species == o.species && order == o.order; }
+};
+
+struct FlatModel {
+    std::vector<std::string> alphabet;
+    std::vector<std::string> names;              // [S]
+    std::vector<int32_t> x0;                     // [S]
+    std::vector<double> rates;                   // [M]
+    std::vector<std::vector<Reactant>> reactants;  // [M], ascending species
+    std::vector<std::vector<int32_t>> delta;     // [M][S]
+    std::vector<int32_t> rule_of;                // [M]
+    int32_t n_rules = 0;
+    int64_t x_cap_max = 0;                       // largest cap with every prod C(cap, r) < 2^53
+
+    int32_t S() const { return (int32_t)names.size(); }
+    int32_t M() const { return (int32_t)rates.size(); }
+};
+
+// Parse + flatten.  Throws cwc::Error with CWC_E_INVALID / CWC_E_PARSE / CWC_E_UNSUPPORTED.
+FlatModel compile_model(const std::vector<std::string>& alphabet,
+                        const std::vector<std::string>& rules, const std::vector<double>& rates,
+                        const std::string& initial_term);
+
+// Largest cap in [1, limit] such that prod_s C(cap, r_s) < 2^53 for every reaction (R9).
+int64_t max_exact_cap(const std::vector<std::vector<Reactant>>& reactants, int64_t limit);
+
+}  // namespace cwc

@@ -1,0 +1,37 @@
+// cwc_params.h — kernel parameter block shared by the host runtime (runtime.cpp) and the
+// NVRTC-compiled SSA kernel (cwc_ssa.cuh).  Plain C layout, passed by value as
+// __grid_constant__; no includes so NVRTC needs no headers.
+#pragma once
+
+struct cwc_round_keys {
+    unsigned int k0[10];  // key0 + r * 0x9E3779B9, r = 0..9
+    unsigned int k1[10];  // key1 + r * 0xBB67AE85
+};
+
+struct cwc_logtab_entry {
+    double invc, logc, logclo;
+};
+
+struct cwc_params {
+    long long first;            // global id of local instance 0
+    long long count;            // local instances
+    long long K;                // last cut index, T = K + 1
+    double dt;                  // sample_dt, t_k = fl(k * dt)
+    long long n_items;          // work items = n_quanta * count
+    long long qs;               // cuts per quantum (Q/tau)
+    int refill;                 // 1 = global atomic work queue with warp-aggregated refill
+    int pad0;
+    cwc_round_keys rk;          // Philox round keys of the seed
+    unsigned long long* stats;  // packed int64 stats (cwc.h layout)
+    int* raw;                   // [T][S][count] or nullptr
+    int* st_x;                  // [S][count] saved species counts
+    double* st_t;               // [count] saved time
+    unsigned long long* st_step;  // [count] saved step (= reactions applied)
+    long long* st_k;            // [count] next cut index
+    unsigned int* st_flags;     // [count] CWC_FLAG_* | CWC_TERMINAL
+    unsigned int* st_qdone;     // [count] quanta completed (release/acquire)
+    unsigned long long* work;   // work-queue counter
+    const cwc_logtab_entry* logtab;  // [128]
+};
+
+#define CWC_TERMINAL 0x80000000u

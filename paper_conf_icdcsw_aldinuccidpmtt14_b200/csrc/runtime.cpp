@@ -1,0 +1,508 @@
+// runtime.cpp — NVRTC compilation, device buffers, the simulate launch and host finalisation.
+//
+// One cwc_simulate_range = two async memsets + ONE launch of the persistent SSA kernel on the
+// caller's stream (torch's, when called from Python).  Everything the hot path computes runs in
+// that kernel; the host only validates, sizes buffers and, at finalize, turns the exact integer
+// accumulators into mean / variance / quantiles (R10, R11).
+#include "runtime.hpp"
+
+#include <nvrtc.h>
+
+#include <algorithm>
+#include <cmath>
+#include <cstdio>
+#include <cstdlib>
+#include <cstring>
+#include <fstream>
+#include <mutex>
+#include <sstream>
+#include <sys/stat.h>
+#include <unistd.h>
+
+#include "cwc.h"
+
+extern const char* const cwc_embedded_params_h;
+extern const char* const cwc_embedded_rng_cuh;
+extern const char* const cwc_embedded_ssa_cuh;
+
+namespace cwc {
+
+// ------------------------------------------------------------------------------------ errors
+[[noreturn]] static void fail(int32_t code, const std::string& msg) { throw Error(code, msg); }
+
+static void ck(cudaError_t e, const char* what) {
+    if (e == cudaSuccess) return;
+    if (e == cudaErrorMemoryAllocation) fail(CWC_E_OOM, std::string(what) + ": " + cudaGetErrorString(e));
+    fail(CWC_E_CUDA, std::string(what) + ": " + cudaGetErrorString(e));
+}
+
+// ------------------------------------------------------------------------------------ driver API
+// Resolved through the runtime (cudaGetDriverEntryPoint) so the library loads on machines
+// without a driver; only simulate needs one.
+struct Driver {
+    CUresult (*ModuleLoadData)(CUmodule*, const void*) = nullptr;
+    CUresult (*ModuleUnload)(CUmodule) = nullptr;
+    CUresult (*ModuleGetFunction)(CUfunction*, CUmodule, const char*) = nullptr;
+    CUresult (*LaunchKernel)(CUfunction, unsigned, unsigned, unsigned, unsigned, unsigned, unsigned, unsigned,
+                             CUstream, void**, void**) = nullptr;
+    CUresult (*FuncGetAttribute)(int*, CUfunction_attribute, CUfunction) = nullptr;
+    CUresult (*Occupancy)(int*, CUfunction, int, size_t) = nullptr;
+    bool ok = false;
+};
+
+static Driver& driver() {
+    static Driver d;
+    static std::once_flag once;
+    std::call_once(once, [] {
+        auto get = [](const char* name, void** fn) {
+            cudaDriverEntryPointQueryResult q;
+            return cudaGetDriverEntryPoint(name, fn, cudaEnableDefault, &q) == cudaSuccess &&
+                   q == cudaDriverEntryPointSuccess && *fn;
+        };
+        d.ok = get("cuModuleLoadData", (void**)&d.ModuleLoadData) &&
+               get("cuModuleUnload", (void**)&d.ModuleUnload) &&
+               get("cuModuleGetFunction", (void**)&d.ModuleGetFunction) &&
+               get("cuLaunchKernel", (void**)&d.LaunchKernel) &&
+               get("cuFuncGetAttribute", (void**)&d.FuncGetAttribute) &&
+               get("cuOccupancyMaxActiveBlocksPerMultiprocessor", (void**)&d.Occupancy);
+    });
+    if (!d.ok) fail(CWC_E_CUDA, "CUDA driver entry points unavailable (no driver / GPU?)");
+    return d;
+}
+
+static void ckd(CUresult r, const char* what) {
+    if (r != CUDA_SUCCESS) fail(CWC_E_CUDA, std::string(what) + ": CUresult " + std::to_string((int)r));
+}
+
+// ------------------------------------------------------------------------------------ sizes
+int64_t grid_K(double t_end, double dt) {
+    if (!(dt > 0) || !std::isfinite(dt)) fail(CWC_E_INVALID, "sample_dt must be > 0");
+    if (!(t_end >= 0) || !std::isfinite(t_end)) fail(CWC_E_INVALID, "t_end must be >= 0");
+    double r = std::nearbyint(t_end / dt);
+    if (r > 2e9) fail(CWC_E_INVALID, "too many sample points");
+    int64_t K = (int64_t)r;
+    if (std::fabs((double)K * dt - t_end) > 1e-9 * std::max(1.0, t_end))
+        fail(CWC_E_INVALID, "t_end is not a multiple of sample_dt");
+    return K;
+}
+
+size_t stats_len(int64_t T, int S, int B) { return (size_t)(T * (1 + 3 * (int64_t)S + (int64_t)S * (B + 2)) + CWC_N_CTR); }
+
+static size_t align256(size_t v) { return (v + 255) & ~(size_t)255; }
+
+struct ScratchLayout {
+    size_t x, t, step, k, flags, qdone, work, total;
+};
+
+static ScratchLayout scratch_layout(int S, int64_t count) {
+    ScratchLayout L{};
+    size_t off = 0;
+    L.x = off; off = align256(off + (size_t)S * count * 4);
+    L.t = off; off = align256(off + (size_t)count * 8);
+    L.step = off; off = align256(off + (size_t)count * 8);
+    L.k = off; off = align256(off + (size_t)count * 8);
+    L.flags = off; off = align256(off + (size_t)count * 4);
+    L.qdone = off; off += (size_t)count * 4;          // qdone and work are contiguous:
+    off = (off + 7) & ~(size_t)7;                     // one memset clears both
+    L.work = off; off = align256(off + 8);
+    L.total = off;
+    return L;
+}
+
+void buffer_sizes(const cwc_model* m, int64_t count, int64_t K, size_t* stats, size_t* raw, size_t* scratch) {
+    const int S = m->fm.S();
+    if (stats) *stats = stats_len(K + 1, S, m->hist_bins);
+    if (raw) *raw = m->raw_samples ? (size_t)(K + 1) * S * (size_t)count : 0;
+    if (scratch) *scratch = scratch_layout(S, count).total;
+}
+
+// ------------------------------------------------------------------------------------ NVRTC
+static std::string strip_pragma_once(const char* s) {
+    std::string out(s);
+    size_t p;
+    while ((p = out.find("#pragma once")) != std::string::npos) out.erase(p, 12);
+    return out;
+}
+
+std::string generate_kernel_source(const FlatModel& fm, const KernelConfig& cfg) {
+    std::string src = "// CWC ensemble SSA kernel, generated for one model (NVRTC, sm_100a)\n";
+    src += strip_pragma_once(cwc_embedded_params_h);
+    src += strip_pragma_once(cwc_embedded_rng_cuh);
+    src += generate_model_section(fm, cfg);
+    src += strip_pragma_once(cwc_embedded_ssa_cuh);
+    return src;
+}
+
+static uint64_t fnv1a(const std::string& s) {
+    uint64_t h = 1469598103934665603ULL;
+    for (unsigned char c : s) { h ^= c; h *= 1099511628211ULL; }
+    return h;
+}
+
+static std::string cache_dir() {
+    const char* e = std::getenv("CWC_CACHE_DIR");
+    if (e && *e) return e;
+    const char* home = std::getenv("HOME");
+    return std::string(home && *home ? home : "/tmp") + "/.cache/cwc_b200";
+}
+
+static const char* kNvrtcOpts[] = {"--gpu-architecture=sm_100a", "-fmad=false", "-lineinfo", "-std=c++17",
+                                   "--ptxas-options=-v", "-DCWC_NVRTC=1"};
+
+static void parse_ptxas(cwc_model* m) {
+    m->regs = -1;
+    m->local_bytes = 0;
+    size_t p = m->nvrtc_log.find("Used ");
+    if (p != std::string::npos) m->regs = std::atoi(m->nvrtc_log.c_str() + p + 5);
+    size_t q = m->nvrtc_log.find("bytes spill stores");
+    if (q != std::string::npos) {
+        size_t b = m->nvrtc_log.rfind(',', q);
+        if (b != std::string::npos) m->local_bytes = std::atoi(m->nvrtc_log.c_str() + b + 1);
+    }
+}
+
+void compile(cwc_model* m) {
+    KernelConfig cfg;
+    cfg.block_threads = m->block_threads;
+    cfg.hist_bins = m->hist_bins;
+    cfg.x_cap = m->x_cap;
+    cfg.hist_lo = m->hist_lo;
+    cfg.hist_width = m->hist_width;
+    std::string src = generate_kernel_source(m->fm, cfg);
+    int major = 0, minor = 0;
+    nvrtcVersion(&major, &minor);
+    std::string key = std::to_string(fnv1a(src)) + "-nvrtc" + std::to_string(major) + "." + std::to_string(minor);
+    if (key == m->compiled_key && !m->cubin.empty()) return;
+
+    std::vector<char> cubin;
+    std::string log;
+    const std::string dir = cache_dir();
+    const std::string path = dir + "/" + key + ".cubin", lpath = dir + "/" + key + ".log";
+    {
+        std::ifstream f(path, std::ios::binary);
+        if (f) {
+            cubin.assign(std::istreambuf_iterator<char>(f), std::istreambuf_iterator<char>());
+            std::ifstream lf(lpath);
+            if (lf) log.assign(std::istreambuf_iterator<char>(lf), std::istreambuf_iterator<char>());
+        }
+    }
+    if (cubin.empty()) {
+        nvrtcProgram prog;
+        if (nvrtcCreateProgram(&prog, src.c_str(), "cwc_ssa.cu", 0, nullptr, nullptr) != NVRTC_SUCCESS)
+            fail(CWC_E_CUDA, "nvrtcCreateProgram failed");
+        nvrtcResult r = nvrtcCompileProgram(prog, (int)(sizeof kNvrtcOpts / sizeof kNvrtcOpts[0]), kNvrtcOpts);
+        size_t ls = 0;
+        nvrtcGetProgramLogSize(prog, &ls);
+        log.assign(ls, '\0');
+        if (ls) nvrtcGetProgramLog(prog, &log[0]);
+        if (!log.empty() && log.back() == '\0') log.pop_back();
+        if (r != NVRTC_SUCCESS) {
+            nvrtcDestroyProgram(&prog);
+            m->nvrtc_log = log;
+            fail(CWC_E_CUDA, "NVRTC compilation failed: " + log.substr(0, 2000));
+        }
+        size_t cs = 0;
+        nvrtcGetCUBINSize(prog, &cs);
+        cubin.resize(cs);
+        nvrtcGetCUBIN(prog, cubin.data());
+        nvrtcDestroyProgram(&prog);
+        // best-effort disk cache
+        std::string cmd = dir;
+        for (size_t i = 1; i <= cmd.size(); ++i)
+            if (i == cmd.size() || cmd[i] == '/') mkdir(cmd.substr(0, i).c_str(), 0755);
+        std::string tmp = path + ".tmp." + std::to_string((long)getpid());
+        {
+            std::ofstream f(tmp, std::ios::binary);
+            if (f) f.write(cubin.data(), (std::streamsize)cubin.size());
+        }
+        std::rename(tmp.c_str(), path.c_str());
+        std::ofstream lf(lpath);
+        if (lf) lf << log;
+    }
+    if (m->module && driver().ok) driver().ModuleUnload(m->module);
+    m->module = nullptr;
+    m->function = nullptr;
+    m->module_device = -1;
+    m->source = src;
+    m->nvrtc_log = log;
+    m->cubin = std::move(cubin);
+    m->compiled_key = key;
+    parse_ptxas(m);
+}
+
+// ------------------------------------------------------------------------------------ device
+static int current_device(cwc_model* m) {
+    int dev = m->device;
+    if (dev < 0) ck(cudaGetDevice(&dev), "cudaGetDevice");
+    ck(cudaSetDevice(dev), "cudaSetDevice");
+    ck(cudaFree(nullptr), "CUDA context init");
+    return dev;
+}
+
+static void ensure_module(cwc_model* m, int dev) {
+    if (m->module && m->module_device == dev) return;
+    Driver& d = driver();
+    if (m->module) d.ModuleUnload(m->module);
+    m->module = nullptr;
+    ckd(d.ModuleLoadData(&m->module, m->cubin.data()), "cuModuleLoadData");
+    ckd(d.ModuleGetFunction(&m->function, m->module, "cwc_ssa_kernel"), "cuModuleGetFunction");
+    m->module_device = dev;
+    int v = 0;
+    if (d.FuncGetAttribute(&v, CU_FUNC_ATTRIBUTE_NUM_REGS, m->function) == CUDA_SUCCESS) m->regs = v;
+    if (d.FuncGetAttribute(&v, CU_FUNC_ATTRIBUTE_LOCAL_SIZE_BYTES, m->function) == CUDA_SUCCESS) m->local_bytes = v;
+    if (d.FuncGetAttribute(&v, CU_FUNC_ATTRIBUTE_MAX_THREADS_PER_BLOCK, m->function) == CUDA_SUCCESS) m->max_threads = v;
+}
+
+static void free_owned(cwc_model* m) {
+    if (!m->bound) {
+        if (m->d_stats) cudaFree(m->d_stats);
+        if (m->d_raw) cudaFree(m->d_raw);
+        if (m->d_scratch) cudaFree(m->d_scratch);
+    }
+    m->d_stats = nullptr; m->d_raw = nullptr; m->d_scratch = nullptr;
+    m->stats_cap = m->raw_cap = m->scratch_cap = 0;
+}
+
+void bind_buffers(cwc_model* m, int64_t* stats, size_t stats_n, int32_t* raw, size_t raw_n, void* scratch,
+                  size_t scratch_bytes) {
+    free_owned(m);
+    if (!stats && !raw && !scratch) {
+        m->bound = false;
+        return;
+    }
+    if (!stats || !scratch) fail(CWC_E_INVALID, "stats and scratch buffers are required when binding");
+    m->bound = true;
+    m->d_stats = stats;
+    m->stats_cap = stats_n * 8;
+    m->d_raw = raw;
+    m->raw_cap = raw ? raw_n * 4 : 0;
+    m->d_scratch = scratch;
+    m->scratch_cap = scratch_bytes;
+}
+
+template <class T>
+static void grow(T*& p, size_t& cap, size_t need_bytes, const char* what) {
+    if (cap >= need_bytes && p) return;
+    if (p) cudaFree(p);
+    p = nullptr;
+    cap = 0;
+    void* q = nullptr;
+    ck(cudaMalloc(&q, std::max<size_t>(need_bytes, 256)), what);
+    p = (T*)q;
+    cap = need_bytes;
+}
+
+void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count, double t_end, double dt,
+                    uint64_t seed, cudaStream_t stream) {
+    if (n_total <= 0) fail(CWC_E_INVALID, "n_total must be > 0");
+    if (first < 0 || count < 0 || first + count > n_total) fail(CWC_E_INVALID, "instance range outside [0, n_total)");
+    const int64_t K = grid_K(t_end, dt);
+    const int64_t T = K + 1;
+    const int S = m->fm.S();
+    compile(m);
+    const int dev = current_device(m);
+    ensure_module(m, dev);
+    Driver& d = driver();
+
+    size_t need_stats, need_raw, need_scratch;
+    buffer_sizes(m, count, K, &need_stats, &need_raw, &need_scratch);
+    if (m->bound) {
+        if (m->stats_cap < need_stats * 8 || m->scratch_cap < need_scratch || (need_raw && m->raw_cap < need_raw * 4))
+            fail(CWC_E_INVALID, "bound device buffers too small (see cwc_buffer_sizes)");
+    } else {
+        grow(m->d_stats, m->stats_cap, need_stats * 8, "cudaMalloc(stats)");
+        if (need_raw) grow(m->d_raw, m->raw_cap, need_raw * 4, "cudaMalloc(raw)");
+        grow(m->d_scratch, m->scratch_cap, need_scratch, "cudaMalloc(scratch)");
+    }
+    if (!m->d_logtab || m->logtab_device != dev) {
+        if (m->d_logtab) cudaFree(m->d_logtab);
+        m->d_logtab = nullptr;
+        cwc_logtab_entry tab[128];
+        build_log_table(tab);
+        ck(cudaMalloc(&m->d_logtab, sizeof tab), "cudaMalloc(logtab)");
+        ck(cudaMemcpy(m->d_logtab, tab, sizeof tab, cudaMemcpyHostToDevice), "upload logtab");
+        m->logtab_device = dev;
+    }
+    if (!stream) {
+        if (!m->own_stream) ck(cudaStreamCreateWithFlags(&m->own_stream, cudaStreamNonBlocking), "cudaStreamCreate");
+        stream = m->own_stream;
+    }
+    if (!m->ev0) {
+        ck(cudaEventCreate(&m->ev0), "cudaEventCreate");
+        ck(cudaEventCreate(&m->ev1), "cudaEventCreate");
+    }
+
+    // launch geometry: persistent grid of (SMs x resident CTAs), no more lanes than instances
+    int sms = 0;
+    ck(cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev), "SM count");
+    int occ = 0;
+    ckd(d.Occupancy(&occ, m->function, m->block_threads, 0), "occupancy");
+    if (occ < 1) fail(CWC_E_CUDA, "kernel cannot be resident with block_threads = " + std::to_string(m->block_threads));
+    int per_sm = m->blocks_per_sm > 0 ? std::min(m->blocks_per_sm, occ) : occ;
+    int64_t grid = (int64_t)sms * per_sm;
+    grid = std::min<int64_t>(grid, std::max<int64_t>(1, (count + m->block_threads - 1) / m->block_threads));
+    const int64_t lanes = grid * m->block_threads;
+    int64_t qs;
+    if (!m->refill) qs = T;  // static assignment: whole trajectories (no cross-lane dependencies)
+    else if (m->quantum_samples > 0) qs = std::min<int64_t>(m->quantum_samples, T);
+    else qs = (count >= 4 * lanes) ? (T + 7) / 8 : T;
+    const int64_t nq = (T + qs - 1) / qs;
+
+    const ScratchLayout L = scratch_layout(S, count);
+    char* sc = (char*)m->d_scratch;
+    cwc_params P;
+    std::memset(&P, 0, sizeof P);
+    P.first = first;
+    P.count = count;
+    P.K = K;
+    P.dt = dt;
+    P.n_items = nq * count;
+    P.qs = qs;
+    P.refill = m->refill;
+    const uint32_t key0 = (uint32_t)seed, key1 = (uint32_t)(seed >> 32);
+    for (int r = 0; r < 10; ++r) {
+        P.rk.k0[r] = key0 + (uint32_t)r * 0x9E3779B9u;
+        P.rk.k1[r] = key1 + (uint32_t)r * 0xBB67AE85u;
+    }
+    P.stats = (unsigned long long*)m->d_stats;
+    P.raw = need_raw ? m->d_raw : nullptr;
+    P.st_x = (int*)(sc + L.x);
+    P.st_t = (double*)(sc + L.t);
+    P.st_step = (unsigned long long*)(sc + L.step);
+    P.st_k = (long long*)(sc + L.k);
+    P.st_flags = (unsigned int*)(sc + L.flags);
+    P.st_qdone = (unsigned int*)(sc + L.qdone);
+    P.work = (unsigned long long*)(sc + L.work);
+    P.logtab = m->d_logtab;
+
+    ck(cudaMemsetAsync(m->d_stats, 0, need_stats * 8, stream), "memset(stats)");
+    ck(cudaMemsetAsync(sc + L.qdone, 0, L.work + 8 - L.qdone, stream), "memset(queue)");
+    ck(cudaEventRecord(m->ev0, stream), "cudaEventRecord");
+    if (count > 0) {
+        void* args[] = {&P};
+        ckd(d.LaunchKernel(m->function, (unsigned)grid, 1, 1, (unsigned)m->block_threads, 1, 1, 0, (CUstream)stream,
+                           args, nullptr),
+            "cuLaunchKernel");
+    }
+    ck(cudaEventRecord(m->ev1, stream), "cudaEventRecord");
+    ck(cudaGetLastError(), "launch");
+
+    m->simulated = true;
+    m->finalized = false;
+    m->last_stream = stream;
+    m->n_total = n_total;
+    m->first = first;
+    m->count = count;
+    m->K = K;
+    m->dt = dt;
+    m->t_end = t_end;
+    m->seed = seed;
+    m->last_stats_len = need_stats;
+    m->items = nq * count;
+    m->qs = qs;
+    m->grid = (int)grid;
+}
+
+// ------------------------------------------------------------------------------------ finalize
+static double quantile_from_hist(const int64_t* h, int B, int64_t n, double q, int64_t lo, int64_t w) {
+    if (n == 0) return NAN;
+    int64_t need = (int64_t)std::ceil(q * (double)n);
+    if (need < 1) need = 1;
+    int64_t c = 0;
+    for (int b = 0; b < B + 2; ++b) {
+        c += h[b];
+        if (c >= need) {
+            if (b == 0) return -INFINITY;
+            if (b == B + 1) return INFINITY;
+            return (double)(lo + w * (int64_t)(b - 1));
+        }
+    }
+    return INFINITY;
+}
+
+void finalize(cwc_model* m, const int64_t* host_stats) {
+    if (!m->simulated) fail(CWC_E_STATE, "no simulation to finalize");
+    const int64_t T = m->K + 1;
+    const int S = m->fm.S(), B = m->hist_bins;
+    const size_t len = m->last_stats_len;
+    m->h_stats.resize(len);
+    ck(cudaStreamSynchronize(m->last_stream), "simulation");
+    float ms = 0;
+    if (cudaEventElapsedTime(&ms, m->ev0, m->ev1) == cudaSuccess) m->kernel_ms = ms;
+    if (host_stats) std::memcpy(m->h_stats.data(), host_stats, len * 8);
+    else ck(cudaMemcpy(m->h_stats.data(), m->d_stats, len * 8, cudaMemcpyDeviceToHost), "copy stats");
+
+    const int64_t* p = m->h_stats.data();
+    const int64_t TS = T * S;
+    m->h_n.assign(p, p + T);
+    m->h_sum.assign(p + T, p + T + TS);
+    m->h_sqlo.assign(p + T + TS, p + T + 2 * TS);
+    m->h_sqhi.assign(p + T + 2 * TS, p + T + 3 * TS);
+    m->h_hist.assign(p + T + 3 * TS, p + T + 3 * TS + TS * (B + 2));
+    m->times.resize(T);
+    m->mean.assign(TS, NAN);
+    m->var.assign(TS, NAN);
+    m->sumsq_d.resize(TS);
+    const int nq = (int)m->quantiles.size();
+    m->quant.assign(TS * nq, NAN);
+    for (int64_t k = 0; k < T; ++k) {
+        m->times[k] = (double)k * m->dt;
+        const int64_t n = m->h_n[k];
+        for (int s = 0; s < S; ++s) {
+            const int64_t i = k * S + s;
+            const __int128 sum = m->h_sum[i];
+            const __int128 sq = ((__int128)(uint64_t)m->h_sqhi[i] << 32) + (__int128)(uint64_t)m->h_sqlo[i];
+            m->sumsq_d[i] = (double)sq;
+            if (n > 0) m->mean[i] = (double)sum / (double)n;
+            if (n > 1) m->var[i] = (double)((__int128)n * sq - sum * sum) / (double)((__int128)n * (n - 1));
+            for (int qi = 0; qi < nq; ++qi)
+                m->quant[i * nq + qi] = quantile_from_hist(&m->h_hist[i * (B + 2)], B, n, m->quantiles[qi],
+                                                           m->hist_lo[s], m->hist_width[s]);
+        }
+    }
+    m->finalized = true;
+}
+
+void copy_samples(cwc_model* m, int64_t first, int64_t count, int32_t* out) {
+    if (!m->simulated) fail(CWC_E_STATE, "no simulation");
+    if (!m->raw_samples || !m->d_raw) fail(CWC_E_STATE, "raw samples are disabled");
+    if (first < 0 || count < 0 || first + count > m->count) fail(CWC_E_INVALID, "range outside the last simulation");
+    if (!out) fail(CWC_E_INVALID, "null output");
+    ck(cudaStreamSynchronize(m->last_stream), "simulation");
+    if (count == 0) return;
+    const size_t rows = (size_t)(m->K + 1) * m->fm.S();
+    ck(cudaMemcpy2D(out, (size_t)count * 4, m->d_raw + first, (size_t)m->count * 4, (size_t)count * 4, rows,
+                    cudaMemcpyDeviceToHost),
+       "copy samples");
+}
+
+void copy_records(cwc_model* m, int64_t first, int64_t count, uint8_t* flags, int64_t* reactions, double* t_last) {
+    if (!m->simulated) fail(CWC_E_STATE, "no simulation");
+    if (first < 0 || count < 0 || first + count > m->count) fail(CWC_E_INVALID, "range outside the last simulation");
+    ck(cudaStreamSynchronize(m->last_stream), "simulation");
+    if (count == 0) return;
+    const ScratchLayout L = scratch_layout(m->fm.S(), m->count);
+    const char* sc = (const char*)m->d_scratch;
+    if (flags) {
+        std::vector<uint32_t> f(count);
+        ck(cudaMemcpy(f.data(), sc + L.flags + first * 4, count * 4, cudaMemcpyDeviceToHost), "copy flags");
+        for (int64_t i = 0; i < count; ++i) flags[i] = (uint8_t)(f[i] & 3u);
+    }
+    if (reactions)
+        ck(cudaMemcpy(reactions, sc + L.step + first * 8, count * 8, cudaMemcpyDeviceToHost), "copy reactions");
+    if (t_last) ck(cudaMemcpy(t_last, sc + L.t + first * 8, count * 8, cudaMemcpyDeviceToHost), "copy times");
+}
+
+}  // namespace cwc
+
+cwc_model::~cwc_model() {
+    if (module) {
+        cwc::Driver& d = cwc::driver();
+        d.ModuleUnload(module);
+    }
+    cwc::free_owned(this);
+    if (d_logtab) cudaFree(d_logtab);
+    if (own_stream) cudaStreamDestroy(own_stream);
+    if (ev0) cudaEventDestroy(ev0);
+    if (ev1) cudaEventDestroy(ev1);
+}

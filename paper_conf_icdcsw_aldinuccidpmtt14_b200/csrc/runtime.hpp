@@ -1,0 +1,93 @@
+// runtime.hpp — the model handle behind cwc_model_t and its device-side runtime.
+#pragma once
+
+#include <cuda.h>
+#include <cuda_runtime.h>
+
+#include <string>
+#include <vector>
+
+#include "codegen.hpp"
+#include "compiler.hpp"
+#include "device/cwc_params.h"
+
+struct cwc_model {
+    cwc::FlatModel fm;
+
+    // options (cwc.h)
+    int64_t x_cap = 0;
+    int raw_samples = 1;
+    int hist_bins = 256;
+    std::vector<int64_t> hist_lo, hist_width;
+    int64_t quantum_samples = 0;
+    int block_threads = 256;
+    int blocks_per_sm = 0;
+    int refill = 1;
+    int device = -1;
+    std::vector<double> quantiles{0.05, 0.25, 0.5, 0.75, 0.95};
+
+    // flat-view storage for cwc_model_info
+    std::vector<const char*> name_ptrs;
+    std::vector<int32_t> info_nreact, info_rspecies, info_rorder, info_delta;
+
+    // compiled kernel
+    std::string source, nvrtc_log, compiled_key;
+    std::vector<char> cubin;
+    int regs = -1, local_bytes = -1, max_threads = -1;
+    CUmodule module = nullptr;
+    CUfunction function = nullptr;
+    int module_device = -1;
+
+    // device buffers (owned or bound)
+    int64_t* d_stats = nullptr;
+    size_t stats_cap = 0;
+    int32_t* d_raw = nullptr;
+    size_t raw_cap = 0;
+    void* d_scratch = nullptr;
+    size_t scratch_cap = 0;
+    bool bound = false;
+    cwc_logtab_entry* d_logtab = nullptr;
+    int logtab_device = -1;
+    cudaStream_t own_stream = nullptr;
+    cudaEvent_t ev0 = nullptr, ev1 = nullptr;
+
+    // last simulated geometry
+    bool simulated = false;
+    cudaStream_t last_stream = nullptr;
+    int64_t n_total = 0, first = 0, count = 0, K = 0;
+    double dt = 0, t_end = 0;
+    uint64_t seed = 0;
+    size_t last_stats_len = 0;
+    int64_t items = 0, qs = 0;
+    int grid = 0;
+
+    // host results (cwc_stats)
+    bool finalized = false;
+    std::vector<int64_t> h_stats;
+    std::vector<double> times, mean, var, sumsq_d, quant;
+    std::vector<int64_t> h_n, h_sum, h_sqlo, h_sqhi, h_hist;
+    double kernel_ms = 0;
+
+    ~cwc_model();
+};
+
+namespace cwc {
+
+size_t stats_len(int64_t T, int S, int B);
+void buffer_sizes(const cwc_model* m, int64_t count, int64_t K, size_t* stats, size_t* raw, size_t* scratch);
+void compile(cwc_model* m);  // NVRTC (no GPU needed)
+void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count, double t_end, double dt,
+                    uint64_t seed, cudaStream_t stream);
+void finalize(cwc_model* m, const int64_t* host_stats);
+void bind_buffers(cwc_model* m, int64_t* stats, size_t stats_n, int32_t* raw, size_t raw_n, void* scratch,
+                  size_t scratch_bytes);
+void copy_samples(cwc_model* m, int64_t first, int64_t count, int32_t* out);
+void copy_records(cwc_model* m, int64_t first, int64_t count, uint8_t* flags, int64_t* reactions, double* t_last);
+int64_t grid_K(double t_end, double dt);  // R13, throws CWC_E_INVALID
+
+void selftest_philox(int64_t n, const uint32_t* ctr, const uint32_t* key, uint32_t* out);
+void selftest_log(int64_t n, const double* x, double* out);
+void selftest_u01(int64_t n, const uint32_t* words, double* out);
+void build_log_table(cwc_logtab_entry* tab);
+
+}  // namespace cwc

@@ -1,0 +1,148 @@
+"""CPU-side checks of the C ABI library (no GPU): it loads, exports every symbol include/cwc.h
+declares, its rule compiler agrees with the oracle's independent flattening on every workload,
+it rejects what DESIGN.md §3 says it must reject with the right status, and NVRTC compiles the
+model-specialised SSA kernel for sm_100a without spilling.
+"""
+import ctypes
+import os
+import re
+
+import pytest
+
+import workloads as W
+from oracle.cwc_terms import CWCError as OracleError
+from oracle.cwc_terms import flatten, flatten_def
+
+import paper_conf_icdcsw_aldinuccidpmtt14_b200 as cwc
+from paper_conf_icdcsw_aldinuccidpmtt14_b200 import _lib
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+
+
+def _declared_functions():
+    with open(os.path.join(ROOT, "include", "cwc.h")) as f:
+        text = f.read()
+    text = re.sub(r"/\*.*?\*/", "", text, flags=re.S)
+    return sorted(set(re.findall(r"\b(cwc_[a-z0-9_]+)\s*\(", text)))
+
+
+def test_library_exports_every_declared_symbol():
+    so = ctypes.CDLL(_lib.SO_PATH)
+    names = _declared_functions()
+    assert len(names) >= 20
+    for n in names:
+        assert hasattr(so, n), n
+    assert set(names) == set(_lib.SIGNATURES), "binding and header disagree"
+    assert b"sm_100a" in _lib.lib.cwc_version()
+
+
+@pytest.mark.parametrize("name", sorted(W.MODELS) + sorted(W.TINY_MODELS))
+def test_compiler_matches_oracle_flattening(name):
+    md = W.MODELS.get(name) or W.TINY_MODELS[name]
+    m = cwc.Model.from_def(md)
+    info = m.info()
+    fm = flatten_def(md)
+    assert info["names"] == fm.names
+    assert info["x0"] == fm.x0
+    assert info["rates"] == fm.rates
+    assert info["reactants"] == [list(r) for r in fm.reactants]
+    assert info["delta"] == fm.delta
+    assert info["rule_of"] == fm.rule_of
+    assert info["x_cap"] == fm.x_cap
+    assert info["n_rules"] == len(md.rules)
+
+
+REJECT = [
+    (["top: Q -> ."], [1.0], "A", 1),
+    (["top: A ."], [1.0], "A", 2),
+    (["A -> ."], [1.0], "A", 2),
+    (["top: A -> ."], [-1.0], "A", 1),
+    (["top: A -> ."], [float("nan")], "A", 1),
+    (["top: A -> ."], [float("inf")], "A", 1),
+    (["top: A -> (. $x | $X)^c"], [1.0], "A", 3),
+    (["top: (. $x | $X)^c -> ."], [1.0], "A (.|.)^c", 3),
+    (["top: A A A A -> ."], [1.0], "A", 3),
+    (["top: (A | $X)^c -> (. | $X)^c"], [1.0], "A (A|.)^c", 3),
+    (["top: (. $x | $X)^c (. $y | $Y)^c -> (. $y | $X)^c (. $x | $Y)^c"], [1.0], "(.|.)^c (.|.)^c", 3),
+    (["top: A -> B"], [1.0], "(A | .)^top", 1),
+    (["top: A -> B"], [1.0], "(A | .", 2),
+    (["top: A -> B"], [1.0], "3 A", 2),
+]
+
+
+@pytest.mark.parametrize("rules,rates,term,status", REJECT)
+def test_rejections_match_oracle(rules, rates, term, status):
+    with pytest.raises(cwc.CWCError) as e:
+        cwc.Model(["A", "B"], rules, rates, term)
+    assert e.value.status == status, str(e.value)
+    kind = {1: "invalid", 2: "parse", 3: "unsupported"}[status]
+    with pytest.raises(OracleError) as oe:
+        flatten(["A", "B"], rules, rates, term)
+    assert oe.value.kind == kind
+
+
+def test_options_validation():
+    m = cwc.Model.from_def(W.SCHLOGL)
+    cap = m.info()["x_cap_max"]
+    with pytest.raises(cwc.CWCError):
+        m.set_option("x_cap", cap + 1)
+    with pytest.raises(cwc.CWCError):
+        m.set_option("x_cap", 100)          # below x0 = 250
+    with pytest.raises(cwc.CWCError):
+        m.set_option("nope", 1)
+    with pytest.raises(cwc.CWCError):
+        m.set_option("block_threads", 100)
+    with pytest.raises(cwc.CWCError):
+        m.set_option("hist_width.Q", 2)
+    m.set_option("hist_width.X", 4)
+    m.set_option("hist_lo", -3)
+    assert m.info()["hist_width"] == [4] and m.info()["hist_lo"] == [-3]
+    with pytest.raises(cwc.CWCError):
+        m.set_quantiles([0.5, 1.5])
+
+
+def test_state_errors_before_simulate():
+    m = cwc.Model.from_def(W.IMM_DEATH)
+    with pytest.raises(cwc.CWCError) as e:
+        m.stats()
+    assert e.value.status == 6
+    with pytest.raises(cwc.CWCError) as e:
+        m.samples(0, 1)
+    assert e.value.status == 6
+    with pytest.raises(cwc.CWCError) as e:
+        m.buffer_sizes(10, 1.05, 0.1)
+    assert e.value.status == 1
+
+
+def test_buffer_sizes_layout():
+    m = cwc.Model.from_def(W.LOTKA_VOLTERRA, hist_bins=1024)
+    n_stats, n_raw, n_scratch = m.buffer_sizes(1000, 50.0, 0.1)
+    T, S, B = 501, 2, 1024
+    assert n_stats == T * (1 + 3 * S + S * (B + 2)) + _lib.N_CTR
+    assert n_raw == T * S * 1000
+    assert n_scratch >= 1000 * (S * 4 + 8 + 8 + 8 + 4 + 4)
+    m.set_option("raw_samples", 0)
+    assert m.buffer_sizes(1000, 50.0, 0.1)[1] == 0
+
+
+@pytest.mark.parametrize("name", sorted(W.MODELS))
+def test_nvrtc_compiles_for_sm100a_without_spills(name):
+    m = cwc.Model.from_def(W.MODELS[name])
+    src, log = m.compile()
+    assert "cwc_ssa_kernel" in src and "__dmul_rn" in src
+    attrs = m.kernel_attributes()
+    assert attrs["local_bytes"] == 0, log
+    assert 0 < attrs["registers"] <= 255
+    # the species state is indexed by compile-time constants only
+    body = src[src.index("generated model section"):]
+    assert "x[j]" not in body and "x[s]" not in body.split("cwc_bin")[0]
+
+
+def test_simulate_without_gpu_fails_loudly():
+    torch = pytest.importorskip("torch")
+    if torch.cuda.is_available():
+        pytest.skip("a GPU is present")
+    m = cwc.Model.from_def(W.IMM_DEATH)
+    with pytest.raises(cwc.CWCError) as e:
+        m.simulate(10, 1.0, 1.0, 1)
+    assert e.value.status == 4

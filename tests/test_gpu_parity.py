@@ -1,0 +1,180 @@
+"""GPU parity: the CUDA path (through the C ABI) against the oracle, element by element.
+
+Bar (north_star): integer species counts at every cut identical to the oracle
+(we require 100 %: both sides follow R3-R7 bit for bit), identical per-instance flags and
+reaction counts, and finalised statistics bit-identical to the oracle's statistics of the
+oracle's samples.  Sizes span several CTAs and a ragged tail; the bench-size runs are checked
+on sampled instances plus the raw-vs-stats property that holds at any size.
+"""
+import numpy as np
+import pytest
+
+import oracle
+import workloads as W
+from oracle.cwc_terms import flatten_def
+
+from helpers import assert_matches_oracle_stats, assert_stats_match_raw, gpu_run
+
+pytestmark = pytest.mark.gpu
+
+QS = (0.05, 0.25, 0.5, 0.75, 0.95)
+
+
+def _oracle(md, first, count, t_end, dt, seed, nthreads=16):
+    return oracle.simulate(flatten_def(md), first, count, t_end, dt, seed, nthreads=nthreads)
+
+
+# ------------------------------------------------------------------ device primitives
+def test_device_philox_matches_oracle():
+    from paper_conf_icdcsw_aldinuccidpmtt14_b200 import selftest_philox
+    rng = np.random.default_rng(1)
+    n = 50000
+    ctr = rng.integers(0, 2 ** 32, size=(n, 4), dtype=np.uint64).astype(np.uint32)
+    key = rng.integers(0, 2 ** 32, size=(n, 2), dtype=np.uint64).astype(np.uint32)
+    ctr[0], key[0] = 0, 0
+    ctr[1], key[1] = 0xFFFFFFFF, 0xFFFFFFFF
+    ctr[2], key[2] = [0x243F6A88, 0x85A308D3, 0x13198A2E, 0x03707344], [0xA4093822, 0x299F31D0]
+    out = selftest_philox(ctr, key)
+    assert list(out[0]) == [0x6627E8D5, 0xE169C58D, 0xBC57AC4C, 0x9B00DBD8]
+    for i in range(0, n, 97):
+        assert tuple(int(v) for v in out[i]) == oracle.philox4x32_10([int(v) for v in ctr[i]],
+                                                                    [int(v) for v in key[i]])
+
+
+def test_device_u01_matches_oracle():
+    from paper_conf_icdcsw_aldinuccidpmtt14_b200 import selftest_u01
+    rng = np.random.default_rng(2)
+    w = rng.integers(0, 2 ** 32, size=(20000, 2), dtype=np.uint64).astype(np.uint32)
+    w[0] = [0, 0]
+    w[1] = [0xFFFFFFFF, 0xFFFFFFFF]
+    out = selftest_u01(w)
+    for i in range(len(w)):
+        assert out[i] == oracle.u01(int(w[i, 0]), int(w[i, 1]))
+
+
+def test_device_log_bit_identical_to_oracle():
+    from paper_conf_icdcsw_aldinuccidpmtt14_b200 import selftest_log
+    rng = np.random.default_rng(3)
+    u = np.concatenate([rng.random(200000), np.exp2(-rng.random(100000) * 53.0),
+                        [2.0 ** -53, 1 - 2.0 ** -53, 0.5, 0.6875, 0.999, 1 - 1 / 256]])
+    u = u[(u >= 2.0 ** -53) & (u < 1.0)]
+    got = selftest_log(u)
+    ref = np.array([oracle.cwclog(float(v)) for v in u])
+    assert np.array_equal(got.view(np.uint64), ref.view(np.uint64))
+
+
+# ------------------------------------------------------------------ whole-path parity
+def _parity(md, n, t_end, dt, seed, *, first=0, hist_bins=256, hist_width=1, **opts):
+    res, raw, flags, reactions, m = gpu_run(md, first + n, first, n, t_end, dt, seed, hist_bins=hist_bins,
+                                            hist_width=hist_width, quantiles=QS, **opts)
+    orun = _oracle(md, first, n, t_end, dt, seed)
+    assert raw.shape == orun.raw.shape
+    same = np.all(raw == orun.raw, axis=(0, 1))
+    assert same.mean() == 1.0, f"{(~same).sum()} of {n} instances differ"
+    assert np.array_equal(flags, orun.flags)
+    assert np.array_equal(reactions, orun.reactions)
+    assert res.reactions == int(orun.reactions.sum())
+    assert res.absorbed == int((orun.flags == oracle.FLAG_ABSORBED).sum())
+    assert res.overflowed == int((orun.flags == oracle.FLAG_OVERFLOWED).sum())
+    assert res.finished == n
+    assert_matches_oracle_stats(res, orun.raw, QS)
+    return res, raw, m
+
+
+def test_config1_imm_death_full():
+    cfg = W.CONFIGS["imm_death"]
+    _parity(cfg.model, cfg.n_instances, cfg.t_end, cfg.sample_dt, cfg.seed, hist_bins=cfg.hist_bins,
+            hist_width=cfg.hist_width)
+
+
+def test_lv_short_horizon_ragged():
+    cfg = W.CONFIGS["lv"]
+    _parity(cfg.model, 1537, 2.0, cfg.sample_dt, cfg.seed, hist_bins=cfg.hist_bins, hist_width=cfg.hist_width)
+
+
+def test_lv_long_horizon_absorb_and_overflow():
+    # long horizon: predator extinction, prey runaway past X_cap (R9) and full extinction (R8)
+    cfg = W.CONFIGS["lv"]
+    res, raw, m = _parity(cfg.model, 300, 50.0, 0.5, cfg.seed + 7, hist_bins=cfg.hist_bins,
+                          hist_width=cfg.hist_width)
+    assert res.overflowed > 0
+
+
+def test_schlogl_small_quanta():
+    cfg = W.CONFIGS["schlogl"]
+    _parity(cfg.model, 3001, 5.0, cfg.sample_dt, cfg.seed, hist_bins=cfg.hist_bins, quantum_samples=3)
+
+
+def test_circadian_small():
+    cfg = W.CONFIGS["circadian"]
+    _parity(cfg.model, 700, 12.0, cfg.sample_dt, cfg.seed, first=123_456, hist_bins=cfg.hist_bins,
+            hist_width=cfg.hist_width)
+
+
+def test_compartments_small():
+    cfg = W.CONFIGS["compartments"]
+    _parity(cfg.model, 900, 20.0, cfg.sample_dt, cfg.seed, hist_bins=cfg.hist_bins)
+
+
+@pytest.mark.parametrize("name", sorted(W.TINY_MODELS))
+def test_tiny_models(name):
+    _parity(W.TINY_MODELS[name], 257, 6.0, 0.25, 99)
+
+
+def test_zero_horizon_and_single_instance():
+    _parity(W.LOTKA_VOLTERRA, 1, 0.0, 0.1, 5)
+    _parity(W.SCHLOGL, 1, 3.0, 0.1, 5)
+
+
+# ------------------------------------------------------------------ schedule invariance (R12)
+def test_schedule_invariance():
+    md = W.SCHLOGL
+    base = None
+    for opts in ({}, {"quantum_samples": 1}, {"quantum_samples": 7}, {"block_threads": 128},
+                 {"block_threads": 512, "quantum_samples": 2}, {"refill": False}, {"blocks_per_sm": 1}):
+        res, raw, flags, reactions, _ = gpu_run(md, 5000, 0, 5000, 4.0, 0.1, 42, hist_bins=512, **opts)
+        cur = (res.n, res.sum, res.sqlo, res.sqhi, res.hist, raw, reactions)
+        if base is None:
+            base = cur
+        else:
+            for a, b in zip(base, cur):
+                assert np.array_equal(a, b), opts
+
+
+def test_sharding_invariance():
+    """Disjoint ranges summed == one run (what the NCCL all-reduce relies on, §8(e))."""
+    md, N, t_end, dt, seed = W.LOTKA_VOLTERRA, 4000, 3.0, 0.1, 7
+    full, raw_full, *_ = gpu_run(md, N, 0, N, t_end, dt, seed, hist_bins=64, hist_width=256)
+    acc = None
+    raws = []
+    import paper_conf_icdcsw_aldinuccidpmtt14_b200 as cwc
+    for a, b in ((0, 1000), (1000, 2999), (2999, 4000)):
+        m = cwc.Model.from_def(md, hist_bins=64, hist_width=256)
+        m.simulate_range(N, a, b - a, t_end, dt, seed)
+        res = m.finalize()
+        raws.append(m.samples(0, b - a))
+        cur = [res.n, res.sum, res.sqlo, res.sqhi, res.hist]
+        acc = cur if acc is None else [x + y for x, y in zip(acc, cur)]
+    for a, b in zip(acc, [full.n, full.sum, full.sqlo, full.sqhi, full.hist]):
+        assert np.array_equal(a, b)
+    assert np.array_equal(np.concatenate(raws, axis=2), raw_full)
+
+
+# ------------------------------------------------------------------ bench-size runs, sampled
+@pytest.mark.parametrize("cname", ["lv", "schlogl"])
+def test_full_size_sampled(cname):
+    cfg = W.CONFIGS[cname]
+    N = cfg.n_instances
+    res, raw, flags, reactions, m = gpu_run(cfg.model, N, 0, N, cfg.t_end, cfg.sample_dt, cfg.seed,
+                                            hist_bins=cfg.hist_bins, hist_width=cfg.hist_width, quantiles=QS)
+    assert res.finished == N
+    assert_stats_match_raw(res, raw)
+    rng = np.random.default_rng(0)
+    pick = sorted(set([0, 1, N - 1] + list(rng.integers(0, N, 29))))
+    fm = flatten_def(cfg.model)
+    cm = oracle.CModel(fm)
+    for i in pick:
+        o = oracle.simulate(cm, i, 1, cfg.t_end, cfg.sample_dt, cfg.seed)
+        assert np.array_equal(raw[:, :, i], o.raw[:, :, 0]), i
+        assert reactions[i] == o.reactions[0] and flags[i] == o.flags[0]
+    assert res.reactions == int(reactions.sum())
