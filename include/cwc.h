@@ -146,11 +146,11 @@ cwc_status cwc_bind_device_buffers(cwc_model_t m, int64_t* stats, size_t stats_l
  * K = llround(t_end/sample_dt) (R7, R13).  Instance i uses the Philox stream keyed by
  * (seed, i) (R3), so any sharding of [0, n_total) gives bit-identical trajectories and
  * statistics.  The packed stats buffer is zeroed and filled by the call.
- * The work is enqueued on cuda_stream (a cudaStream_t; NULL = the handle's own stream) and
+ * The work is enqueued on cuda_stream (a cudaStream_t; NULL = the legacy default stream) and
  * the call returns without waiting; results are valid once the stream has drained
  * (cwc_stats_finalize / cwc_samples / cwc_instance_records synchronise it).
- * cwc_simulate(m, n, t_end, dt, seed) == cwc_simulate_range(m, n, 0, n, ..., NULL) followed
- * by cwc_stats_finalize (synchronous).
+ * cwc_simulate(m, n, t_end, dt, seed) == cwc_simulate_range(m, n, 0, n, ...) on the handle's
+ * own stream followed by cwc_stats_finalize (synchronous).
  * Errors: CWC_E_INVALID (n_total <= 0, count < 0, first+count > n_total, t_end < 0,
  *         sample_dt <= 0, |K*dt - t_end| > 1e-9*max(1,t_end), buffers too small);
  *         CWC_E_OOM; CWC_E_CUDA.

@@ -63,7 +63,7 @@ class Model:
                  *, x_cap: Optional[int] = None, hist_bins: Optional[int] = None, hist_width=None, hist_lo=None,
                  quantiles: Optional[Sequence[float]] = None, raw_samples: bool = True,
                  quantum_samples: int = 0, block_threads: Optional[int] = None, refill: bool = True,
-                 device: Optional[int] = None):
+                 blocks_per_sm: int = 0, device: Optional[int] = None):
         sp = (ctypes.c_char_p * len(species))(*[s.encode() for s in species])
         rl = (ctypes.c_char_p * max(len(rules), 1))(*[r.encode() for r in rules])
         rt = (ctypes.c_double * max(len(rates), 1))(*[float(k) for k in rates])
@@ -90,6 +90,7 @@ class Model:
         if block_threads is not None:
             self.set_option("block_threads", int(block_threads))
         self.set_option("refill", 1 if refill else 0)
+        self.set_option("blocks_per_sm", int(blocks_per_sm))
         if device is not None:
             self.set_option("device", int(device))
 
@@ -172,12 +173,15 @@ class Model:
 
     def simulate_range(self, n_total: int, first: int, count: int, t_end: float, sample_dt: float, seed: int,
                        stream=None) -> None:
-        """Enqueue instances [first, first+count) on ``stream`` (a torch.cuda.Stream, a raw
-        cudaStream_t int, or None for the handle's own stream).  Asynchronous."""
-        if stream is not None and hasattr(stream, "cuda_stream"):
+        """Enqueue instances [first, first+count) on ``stream``: a torch.cuda.Stream, a raw
+        cudaStream_t int, or None for torch's current stream.  Asynchronous."""
+        if stream is None:
+            import torch
+            stream = torch.cuda.current_stream()
+        if hasattr(stream, "cuda_stream"):
             stream = stream.cuda_stream
         check(lib.cwc_simulate_range(self._h, int(n_total), int(first), int(count), float(t_end),
-                                     float(sample_dt), int(seed), ctypes.c_void_p(stream or 0)))
+                                     float(sample_dt), int(seed), ctypes.c_void_p(int(stream))))
 
     def finalize(self, host_stats: Optional[np.ndarray] = None) -> EnsembleResult:
         if host_stats is not None:

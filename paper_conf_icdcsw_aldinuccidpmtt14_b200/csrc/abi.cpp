@@ -239,7 +239,7 @@ cwc_status cwc_simulate_range(cwc_model_t m, int64_t n_total, int64_t first, int
 cwc_status cwc_simulate(cwc_model_t m, int64_t n, double t_end, double dt, uint64_t seed) {
     return guard([&] {
         need(m != nullptr, "NULL model");
-        cwc::simulate_range(m, n, 0, n, t_end, dt, seed, nullptr);
+        cwc::simulate_range(m, n, 0, n, t_end, dt, seed, nullptr, true);
         cwc::finalize(m, nullptr);
     });
 }

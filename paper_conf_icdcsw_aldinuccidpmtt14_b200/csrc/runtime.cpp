@@ -293,7 +293,7 @@ static void grow(T*& p, size_t& cap, size_t need_bytes, const char* what) {
 }
 
 void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count, double t_end, double dt,
-                    uint64_t seed, cudaStream_t stream) {
+                    uint64_t seed, cudaStream_t stream, bool own_stream) {
     if (n_total <= 0) fail(CWC_E_INVALID, "n_total must be > 0");
     if (first < 0 || count < 0 || first + count > n_total) fail(CWC_E_INVALID, "instance range outside [0, n_total)");
     const int64_t K = grid_K(t_end, dt);
@@ -323,7 +323,7 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
         ck(cudaMemcpy(m->d_logtab, tab, sizeof tab, cudaMemcpyHostToDevice), "upload logtab");
         m->logtab_device = dev;
     }
-    if (!stream) {
+    if (own_stream) {
         if (!m->own_stream) ck(cudaStreamCreateWithFlags(&m->own_stream, cudaStreamNonBlocking), "cudaStreamCreate");
         stream = m->own_stream;
     }

@@ -77,7 +77,7 @@ size_t stats_len(int64_t T, int S, int B);
 void buffer_sizes(const cwc_model* m, int64_t count, int64_t K, size_t* stats, size_t* raw, size_t* scratch);
 void compile(cwc_model* m);  // NVRTC (no GPU needed)
 void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count, double t_end, double dt,
-                    uint64_t seed, cudaStream_t stream);
+                    uint64_t seed, cudaStream_t stream, bool own_stream = false);
 void finalize(cwc_model* m, const int64_t* host_stats);
 void bind_buffers(cwc_model* m, int64_t* stats, size_t stats_n, int32_t* raw, size_t raw_n, void* scratch,
                   size_t scratch_bytes);
