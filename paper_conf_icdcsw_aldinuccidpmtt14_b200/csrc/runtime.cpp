@@ -15,6 +15,7 @@
 #include <cstring>
 #include <fstream>
 #include <mutex>
+#include <dlfcn.h>
 #include <sstream>
 #include <sys/stat.h>
 #include <unistd.h>
@@ -146,6 +147,53 @@ static std::string cache_dir() {
     return std::string(home && *home ? home : "/tmp") + "/.cache/cwc_b200";
 }
 
+// NVRTC is loaded at run time (dlopen) from the CUDA toolkit of this image rather than linked
+// statically (106 MB): the library stays small and loads where NVRTC is absent.
+struct Nvrtc {
+    decltype(&::nvrtcVersion) Version = nullptr;
+    decltype(&::nvrtcCreateProgram) CreateProgram = nullptr;
+    decltype(&::nvrtcCompileProgram) CompileProgram = nullptr;
+    decltype(&::nvrtcGetProgramLogSize) GetProgramLogSize = nullptr;
+    decltype(&::nvrtcGetProgramLog) GetProgramLog = nullptr;
+    decltype(&::nvrtcGetCUBINSize) GetCUBINSize = nullptr;
+    decltype(&::nvrtcGetCUBIN) GetCUBIN = nullptr;
+    decltype(&::nvrtcDestroyProgram) DestroyProgram = nullptr;
+    bool ok = false;
+    std::string where;
+};
+
+static Nvrtc& nvrtc() {
+    static Nvrtc n;
+    static std::once_flag once;
+    std::call_once(once, [] {
+        std::vector<std::string> cands;
+        if (const char* e = std::getenv("CWC_NVRTC_PATH")) cands.push_back(e);
+        const char* home = std::getenv("CUDA_HOME");
+        cands.push_back(std::string(home && *home ? home : "/usr/local/cuda") + "/lib64/libnvrtc.so.12");
+        cands.push_back("/usr/local/cuda/lib64/libnvrtc.so.12");
+        cands.push_back("libnvrtc.so.12");
+        void* h = nullptr;
+        for (auto& c : cands) {
+            h = dlopen(c.c_str(), RTLD_NOW | RTLD_LOCAL);
+            if (h) { n.where = c; break; }
+        }
+        if (!h) return;
+        auto sym = [&](const char* s) { return dlsym(h, s); };
+        n.Version = (decltype(n.Version))sym("nvrtcVersion");
+        n.CreateProgram = (decltype(n.CreateProgram))sym("nvrtcCreateProgram");
+        n.CompileProgram = (decltype(n.CompileProgram))sym("nvrtcCompileProgram");
+        n.GetProgramLogSize = (decltype(n.GetProgramLogSize))sym("nvrtcGetProgramLogSize");
+        n.GetProgramLog = (decltype(n.GetProgramLog))sym("nvrtcGetProgramLog");
+        n.GetCUBINSize = (decltype(n.GetCUBINSize))sym("nvrtcGetCUBINSize");
+        n.GetCUBIN = (decltype(n.GetCUBIN))sym("nvrtcGetCUBIN");
+        n.DestroyProgram = (decltype(n.DestroyProgram))sym("nvrtcDestroyProgram");
+        n.ok = n.Version && n.CreateProgram && n.CompileProgram && n.GetProgramLogSize && n.GetProgramLog &&
+               n.GetCUBINSize && n.GetCUBIN && n.DestroyProgram;
+    });
+    if (!n.ok) fail(CWC_E_CUDA, "NVRTC (libnvrtc.so.12) not found; set CWC_NVRTC_PATH");
+    return n;
+}
+
 static const char* kNvrtcOpts[] = {"--gpu-architecture=sm_100a", "-fmad=false", "-lineinfo", "-std=c++17",
                                    "--ptxas-options=-v", "-DCWC_NVRTC=1"};
 
@@ -169,8 +217,9 @@ void compile(cwc_model* m) {
     cfg.hist_lo = m->hist_lo;
     cfg.hist_width = m->hist_width;
     std::string src = generate_kernel_source(m->fm, cfg);
+    Nvrtc& nv = nvrtc();
     int major = 0, minor = 0;
-    nvrtcVersion(&major, &minor);
+    nv.Version(&major, &minor);
     std::string key = std::to_string(fnv1a(src)) + "-nvrtc" + std::to_string(major) + "." + std::to_string(minor);
     if (key == m->compiled_key && !m->cubin.empty()) return;
 
@@ -188,24 +237,24 @@ void compile(cwc_model* m) {
     }
     if (cubin.empty()) {
         nvrtcProgram prog;
-        if (nvrtcCreateProgram(&prog, src.c_str(), "cwc_ssa.cu", 0, nullptr, nullptr) != NVRTC_SUCCESS)
+        if (nv.CreateProgram(&prog, src.c_str(), "cwc_ssa.cu", 0, nullptr, nullptr) != NVRTC_SUCCESS)
             fail(CWC_E_CUDA, "nvrtcCreateProgram failed");
-        nvrtcResult r = nvrtcCompileProgram(prog, (int)(sizeof kNvrtcOpts / sizeof kNvrtcOpts[0]), kNvrtcOpts);
+        nvrtcResult r = nv.CompileProgram(prog, (int)(sizeof kNvrtcOpts / sizeof kNvrtcOpts[0]), kNvrtcOpts);
         size_t ls = 0;
-        nvrtcGetProgramLogSize(prog, &ls);
+        nv.GetProgramLogSize(prog, &ls);
         log.assign(ls, '\0');
-        if (ls) nvrtcGetProgramLog(prog, &log[0]);
+        if (ls) nv.GetProgramLog(prog, &log[0]);
         if (!log.empty() && log.back() == '\0') log.pop_back();
         if (r != NVRTC_SUCCESS) {
-            nvrtcDestroyProgram(&prog);
+            nv.DestroyProgram(&prog);
             m->nvrtc_log = log;
             fail(CWC_E_CUDA, "NVRTC compilation failed: " + log.substr(0, 2000));
         }
         size_t cs = 0;
-        nvrtcGetCUBINSize(prog, &cs);
+        nv.GetCUBINSize(prog, &cs);
         cubin.resize(cs);
-        nvrtcGetCUBIN(prog, cubin.data());
-        nvrtcDestroyProgram(&prog);
+        nv.GetCUBIN(prog, cubin.data());
+        nv.DestroyProgram(&prog);
         // best-effort disk cache
         std::string cmd = dir;
         for (size_t i = 1; i <= cmd.size(); ++i)
