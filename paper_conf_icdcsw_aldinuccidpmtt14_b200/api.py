@@ -63,7 +63,7 @@ class Model:
                  *, x_cap: Optional[int] = None, hist_bins: Optional[int] = None, hist_width=None, hist_lo=None,
                  quantiles: Optional[Sequence[float]] = None, raw_samples: bool = True,
                  quantum_samples: int = 0, block_threads: Optional[int] = None, refill: bool = True,
-                 blocks_per_sm: int = 0, device: Optional[int] = None):
+                 blocks_per_sm: int = 0, device: Optional[int] = None, **options):
         sp = (ctypes.c_char_p * len(species))(*[s.encode() for s in species])
         rl = (ctypes.c_char_p * max(len(rules), 1))(*[r.encode() for r in rules])
         rt = (ctypes.c_double * max(len(rates), 1))(*[float(k) for k in rates])
@@ -91,6 +91,8 @@ class Model:
             self.set_option("block_threads", int(block_threads))
         self.set_option("refill", 1 if refill else 0)
         self.set_option("blocks_per_sm", int(blocks_per_sm))
+        for key, val in options.items():
+            self.set_option(key, int(val))
         if device is not None:
             self.set_option("device", int(device))
 

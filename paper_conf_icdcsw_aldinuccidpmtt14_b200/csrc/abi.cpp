@@ -168,6 +168,12 @@ cwc_status cwc_set_option_i64(cwc_model_t m, const char* key, int64_t v) {
         } else if (k == "block_threads") {
             need(v >= 32 && v <= 1024 && v % 32 == 0, "block_threads: multiple of 32 in [32, 1024]");
             m->block_threads = (int)v;
+        } else if (k == "seed_jit") {
+            need(v == 0 || v == 1, "seed_jit is 0 or 1");
+            m->seed_jit = (int)v;
+        } else if (k == "min_blocks") {
+            need(v >= 0 && v <= 32, "min_blocks in [0, 32]");
+            m->min_blocks = (int)v;
         } else if (k == "blocks_per_sm") {
             need(v >= 0 && v <= 64, "blocks_per_sm in [0, 64]");
             m->blocks_per_sm = (int)v;

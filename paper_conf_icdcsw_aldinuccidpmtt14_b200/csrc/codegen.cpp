@@ -26,8 +26,16 @@ std::string generate_model_section(const FlatModel& fm, const KernelConfig& cfg)
     std::ostringstream o;
     o << "// ---- generated model section: " << S << " species, " << M << " flat reactions\n";
     o << "#define CWC_S " << S << "\n#define CWC_M " << (M > 0 ? M : 1) << "\n#define CWC_B " << cfg.hist_bins
-      << "\n#define CWC_BLOCK " << cfg.block_threads << "\n";
+      << "\n#define CWC_BLOCK " << cfg.block_threads << "\n#define CWC_MINB " << cfg.min_blocks << "\n";
     o << "#define CWC_X_CAP " << cfg.x_cap << "\n\n";
+    if (cfg.seed_keys) {
+        const uint32_t k0 = (uint32_t)cfg.seed, k1 = (uint32_t)(cfg.seed >> 32);
+        o << "#define CWC_STATIC_KEYS 1\nstatic constexpr cwc_round_keys cwc_rk_static = {{";
+        for (int r = 0; r < 10; ++r) o << (r ? ", " : "") << (uint32_t)(k0 + (uint32_t)r * 0x9E3779B9u) << "u";
+        o << "}, {";
+        for (int r = 0; r < 10; ++r) o << (r ? ", " : "") << (uint32_t)(k1 + (uint32_t)r * 0xBB67AE85u) << "u";
+        o << "}};\n\n";
+    }
     for (int s = 0; s < S; ++s) o << "// species " << s << ": " << fm.names[s] << "\n";
 
     // x = x0

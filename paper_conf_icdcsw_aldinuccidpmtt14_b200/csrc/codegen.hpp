@@ -10,7 +10,10 @@ namespace cwc {
 
 struct KernelConfig {
     int block_threads = 256;
+    int min_blocks = 0;  // __launch_bounds__ min blocks per SM (0 = let ptxas choose)
     int hist_bins = 256;
+    bool seed_keys = false;  // bake the Philox round keys of `seed` into the kernel (immediates)
+    uint64_t seed = 0;
     int64_t x_cap = 0;
     std::vector<int64_t> hist_lo, hist_width;  // [S]
 };

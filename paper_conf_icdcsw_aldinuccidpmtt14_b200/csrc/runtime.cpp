@@ -209,14 +209,37 @@ static void parse_ptxas(cwc_model* m) {
     }
 }
 
-void compile(cwc_model* m) {
+void compile(cwc_model* m, const uint64_t* seed) {
     KernelConfig cfg;
     cfg.block_threads = m->block_threads;
+    cfg.min_blocks = m->min_blocks;
     cfg.hist_bins = m->hist_bins;
     cfg.x_cap = m->x_cap;
     cfg.hist_lo = m->hist_lo;
     cfg.hist_width = m->hist_width;
+    if (seed && m->seed_jit) {
+        cfg.seed_keys = true;
+        cfg.seed = *seed;
+    }
     std::string src = generate_kernel_source(m->fm, cfg);
+    // development knob: CWC_KERNEL_DEFINES="A=1;B=2" prepends #defines (kernel variants for A/B
+    // timing); part of the source, hence of the cache key
+    if (const char* e = std::getenv("CWC_KERNEL_DEFINES")) {
+        std::string defs, item;
+        for (const char* p = e;; ++p) {
+            if (*p == ';' || *p == '\0') {
+                size_t eq = item.find('=');
+                if (!item.empty())
+                    defs += "#define " + (eq == std::string::npos ? item : item.substr(0, eq) + " " + item.substr(eq + 1)) +
+                            "\n";
+                item.clear();
+                if (*p == '\0') break;
+            } else {
+                item += *p;
+            }
+        }
+        src = defs + src;
+    }
     Nvrtc& nv = nvrtc();
     int major = 0, minor = 0;
     nv.Version(&major, &minor);
@@ -348,7 +371,7 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     const int64_t K = grid_K(t_end, dt);
     const int64_t T = K + 1;
     const int S = m->fm.S();
-    compile(m);
+    compile(m, &seed);
     const int dev = current_device(m);
     ensure_module(m, dev);
     Driver& d = driver();
@@ -389,7 +412,11 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     if (occ < 1) fail(CWC_E_CUDA, "kernel cannot be resident with block_threads = " + std::to_string(m->block_threads));
     int per_sm = m->blocks_per_sm > 0 ? std::min(m->blocks_per_sm, occ) : occ;
     int64_t grid = (int64_t)sms * per_sm;
-    grid = std::min<int64_t>(grid, std::max<int64_t>(1, (count + m->block_threads - 1) / m->block_threads));
+    // Every resident slot is launched even when there are fewer instances than lanes: warps race
+    // for items on the work queue, so the busy warps spread over all SMs instead of packing the
+    // first CTAs (391 CTAs of 256 on 148 SMs left 35 % of the SMs with 2 CTAs instead of 3).
+    // Only very small ensembles (< 1 warp per CTA) shrink the grid.
+    grid = std::min<int64_t>(grid, std::max<int64_t>(sms, (count + 31) / 32));
     const int64_t lanes = grid * m->block_threads;
     int64_t qs;
     if (!m->refill) qs = T;  // static assignment: whole trajectories (no cross-lane dependencies)

@@ -18,9 +18,11 @@ struct cwc_model {
     int64_t x_cap = 0;
     int raw_samples = 1;
     int hist_bins = 256;
+    int seed_jit = 0;
     std::vector<int64_t> hist_lo, hist_width;
     int64_t quantum_samples = 0;
     int block_threads = 256;
+    int min_blocks = 0;
     int blocks_per_sm = 0;
     int refill = 1;
     int device = -1;
@@ -75,7 +77,7 @@ namespace cwc {
 
 size_t stats_len(int64_t T, int S, int B);
 void buffer_sizes(const cwc_model* m, int64_t count, int64_t K, size_t* stats, size_t* raw, size_t* scratch);
-void compile(cwc_model* m);  // NVRTC (no GPU needed)
+void compile(cwc_model* m, const uint64_t* seed = nullptr);  // NVRTC (no GPU needed)
 void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count, double t_end, double dt,
                     uint64_t seed, cudaStream_t stream, bool own_stream = false);
 void finalize(cwc_model* m, const int64_t* host_stats);

@@ -31,16 +31,19 @@ __global__ void k_philox(int64_t n, const uint32_t* ctr, const uint32_t* key, ui
 }
 
 __global__ void k_log(int64_t n, const double* x, double* out, const cwc_logtab_entry* tab) {
-    __shared__ cwc_logtab_entry s[128];
-    for (int i = threadIdx.x; i < 128; i += blockDim.x) s[i] = tab[i];
+    __shared__ __align__(16) cwc_logsmem s;
+    cwc_logsmem_init(s, tab);
     __syncthreads();
     int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
     if (i < n) out[i] = cwc_log(x[i], s);
 }
 
 __global__ void k_u01(int64_t n, const uint32_t* w, double* out) {
+    __shared__ __align__(16) cwc_logsmem s;
+    if (threadIdx.x == 0) s.k[6] = 0x1.fffffffffffffp-1;  // the constant cwc_logsmem_init stores
+    __syncthreads();
     int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
-    if (i < n) out[i] = cwc_u01(w[2 * i], w[2 * i + 1]);
+    if (i < n) out[i] = cwc_u01(w[2 * i], w[2 * i + 1], s.k[6]);
 }
 
 void ck(cudaError_t e, const char* what) {
