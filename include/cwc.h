@@ -108,7 +108,9 @@ cwc_status cwc_model_info(cwc_model_t m, cwc_model_info_t* out);
  *                        Scheduling only: results are bit-identical for every value (R12).
  *   "block_threads"      CUDA block size (multiple of 32, <= 1024).              default 256
  *   "blocks_per_sm"      persistent CTAs per SM; 0 = occupancy maximum.          default 0
- *   "min_blocks"         register budget: __launch_bounds__ min CTAs per SM; 0 = auto.
+ *   "min_blocks"         register budget: __launch_bounds__ min CTAs per SM; 0 = auto
+ *                        (768 / block_threads, i.e. <= 80 registers).
+ *   "ilp"                1/2 instances interleaved per thread (ablation knob).      default 1
  *   "seed_jit"           0/1: specialise the kernel on the seed (Philox round keys become
  *                        instruction immediates; one NVRTC compile per new seed, cached).
  *   "refill"             0/1: warp-level refill from the global work queue.      default 1

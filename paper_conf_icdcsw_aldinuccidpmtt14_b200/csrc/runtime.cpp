@@ -212,7 +212,10 @@ static void parse_ptxas(cwc_model* m) {
 void compile(cwc_model* m, const uint64_t* seed) {
     KernelConfig cfg;
     cfg.block_threads = m->block_threads;
-    cfg.min_blocks = m->min_blocks;
+    // auto register budget: 768 resident threads per SM (<= 80 registers) — measured best for the
+    // App. B models (fewer, fatter threads lose more to latency than they gain from registers)
+    cfg.min_blocks = m->min_blocks > 0 ? m->min_blocks : std::max(1, 768 / m->block_threads);
+    cfg.ilp = m->ilp;
     cfg.hist_bins = m->hist_bins;
     cfg.x_cap = m->x_cap;
     cfg.hist_lo = m->hist_lo;
@@ -416,8 +419,8 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     // for items on the work queue, so the busy warps spread over all SMs instead of packing the
     // first CTAs (391 CTAs of 256 on 148 SMs left 35 % of the SMs with 2 CTAs instead of 3).
     // Only very small ensembles (< 1 warp per CTA) shrink the grid.
-    grid = std::min<int64_t>(grid, std::max<int64_t>(sms, (count + 31) / 32));
-    const int64_t lanes = grid * m->block_threads;
+    grid = std::min<int64_t>(grid, std::max<int64_t>(sms, (count + 32 * m->ilp - 1) / (32 * m->ilp)));
+    const int64_t lanes = grid * m->block_threads * m->ilp;
     int64_t qs;
     if (!m->refill) qs = T;  // static assignment: whole trajectories (no cross-lane dependencies)
     else if (m->quantum_samples > 0) qs = std::min<int64_t>(m->quantum_samples, T);

@@ -33,3 +33,9 @@ for op, w in ops.most_common(40):
 if "--lines" in sys.argv:
     for w, a, s, smp in sorted(lines, reverse=True)[:int(sys.argv[sys.argv.index('--lines')+1])]:
         print(f"{w/tot_w*100:6.2f}%  {a} {smp:8.0f}  {s}")
+if "--stalls" in sys.argv:
+    n = int(sys.argv[sys.argv.index('--stalls') + 1])
+    tot_s = sum(x[3] for x in lines)
+    print(f"--- top {n} instructions by warp-stall samples (total {tot_s:.0f})")
+    for w, a, s, smp in sorted(lines, key=lambda x: -x[3])[:n]:
+        print(f"{smp/tot_s*100:6.2f}%  {a}  exec {w/tot_w*100:5.2f}%  {s}")

@@ -10,13 +10,15 @@ N = int(sys.argv[2]) if len(sys.argv) > 2 else cfg.n_instances
 opts = dict(a.split("=") for a in sys.argv[3:])
 opts = {k: int(v) for k, v in opts.items()}
 raw = bool(opts.pop("raw", 1))
+t_end = float(opts.pop("t_end", cfg.t_end))
+reps = int(opts.pop("reps", 3))
 m = cwc.Model.from_def(cfg.model, hist_bins=cfg.hist_bins, hist_width=cfg.hist_width, raw_samples=raw, **opts)
-bufs = cwc.DeviceBuffers(m, N, cfg.t_end, cfg.sample_dt)
+bufs = cwc.DeviceBuffers(m, N, t_end, cfg.sample_dt)
 s = torch.cuda.current_stream()
-for it in range(3):
+for it in range(reps):
     e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
     e0.record()
-    m.simulate_range(N, 0, N, cfg.t_end, cfg.sample_dt, cfg.seed, stream=s)
+    m.simulate_range(N, 0, N, t_end, cfg.sample_dt, cfg.seed, stream=s)
     e1.record()
     torch.cuda.synchronize()
     res = m.finalize()
