@@ -283,13 +283,23 @@ def run_b200(args):
     achieved = reactions_per_launch * i_alg / (kern_ms_max / 1e3) / 1e12
     peak = sms * 4 * 32 * f_max / 1e12
     raw_bytes = 0 if args.no_raw else res.n.size * len(info["names"]) * run.count * 4
+    traffic = None   # DRAM bytes per launch from the committed ncu --set full capture of this workload
+    try:
+        with open(os.path.join(ROOT, "profiles", f"traffic_{args.config}.json")) as f:
+            tr = json.load(f)
+        if world == 1 and not args.no_raw and run.count == W.CONFIGS[args.config].n_instances:
+            traffic = tr["dram_bytes_per_launch"]
+    except (OSError, KeyError, ValueError):
+        pass
     roof = {"bound": "alu", "achieved": achieved, "peak": peak, "unit": "Tinst/s", "frac": achieved / peak,
-            "traffic": None,
+            "traffic": traffic,
             "detail": {"algorithmic_inst_per_reaction": i_alg, "sms": sms, "sm_clock_for_peak_mhz": f_max / 1e6,
                        "peak_source": "148 SMs x 4 schedulers x 32 lanes x sm_max_mhz (MEASURED_PEAKS.json)",
                        "frac_at_measured_clock": (achieved / (sms * 128 * clk["sm_mhz"] * 1e6 / 1e12))
                        if clk.get("sm_mhz") else None,
                        "kernel_ms": kern_ms_max,
+                       "algorithmic_bytes_per_launch": raw_bytes + run.buffers.stats.numel() * 8,
+                       "traffic_source": "profiles/traffic_<workload>.json (ncu --set full, dram read+write)",
                        "sample_stream_gbs": (raw_bytes / (kern_ms_max / 1e3) / 1e9) if raw_bytes else 0.0}}
 
     # ---- CPU baseline: the oracle on this host, rank 0 at N = 1 only
