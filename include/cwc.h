@@ -111,6 +111,8 @@ cwc_status cwc_model_info(cwc_model_t m, cwc_model_info_t* out);
  *   "min_blocks"         register budget: __launch_bounds__ min CTAs per SM; 0 = auto
  *                        (768 / block_threads, i.e. <= 80 registers).
  *   "ilp"                1/2 instances interleaved per thread (ablation knob).      default 1
+ *   "smem_stats"         0/1: accumulate n/sum/sumsq per CTA in shared memory and flush once
+ *                        (used when T*(1+3S)*8 bytes fit without lowering residency). default 1
  *   "seed_jit"           0/1: specialise the kernel on the seed (Philox round keys become
  *                        instruction immediates; one NVRTC compile per new seed, cached).
  *   "refill"             0/1: warp-level refill from the global work queue.      default 1

@@ -168,6 +168,9 @@ cwc_status cwc_set_option_i64(cwc_model_t m, const char* key, int64_t v) {
         } else if (k == "block_threads") {
             need(v >= 32 && v <= 1024 && v % 32 == 0, "block_threads: multiple of 32 in [32, 1024]");
             m->block_threads = (int)v;
+        } else if (k == "smem_stats") {
+            need(v == 0 || v == 1, "smem_stats is 0 or 1");
+            m->smem_stats = (int)v;
         } else if (k == "ilp") {
             need(v == 1 || v == 2, "ilp is 1 or 2");
             m->ilp = (int)v;

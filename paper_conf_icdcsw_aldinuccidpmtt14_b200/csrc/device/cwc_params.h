@@ -32,6 +32,8 @@ struct cwc_params {
     unsigned int* st_qdone;     // [count] quanta completed (release/acquire)
     unsigned long long* work;   // work-queue counter
     const cwc_logtab_entry* logtab;  // [128]
+    long long smem_stats;       // 1: n/sum/sumsq accumulate per CTA in dynamic shared memory
+                                //    (T*(1+3S) u64) and are flushed once at the end
 };
 
 #define CWC_TERMINAL 0x80000000u

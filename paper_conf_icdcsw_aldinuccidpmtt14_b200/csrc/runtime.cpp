@@ -48,6 +48,7 @@ struct Driver {
                              CUstream, void**, void**) = nullptr;
     CUresult (*FuncGetAttribute)(int*, CUfunction_attribute, CUfunction) = nullptr;
     CUresult (*Occupancy)(int*, CUfunction, int, size_t) = nullptr;
+    CUresult (*FuncSetAttribute)(CUfunction, CUfunction_attribute, int) = nullptr;
     bool ok = false;
 };
 
@@ -65,7 +66,8 @@ static Driver& driver() {
                get("cuModuleGetFunction", (void**)&d.ModuleGetFunction) &&
                get("cuLaunchKernel", (void**)&d.LaunchKernel) &&
                get("cuFuncGetAttribute", (void**)&d.FuncGetAttribute) &&
-               get("cuOccupancyMaxActiveBlocksPerMultiprocessor", (void**)&d.Occupancy);
+               get("cuOccupancyMaxActiveBlocksPerMultiprocessor", (void**)&d.Occupancy) &&
+               get("cuFuncSetAttribute", (void**)&d.FuncSetAttribute);
     });
     if (!d.ok) fail(CWC_E_CUDA, "CUDA driver entry points unavailable (no driver / GPU?)");
     return d;
@@ -410,9 +412,19 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     // launch geometry: persistent grid of (SMs x resident CTAs), no more lanes than instances
     int sms = 0;
     ck(cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev), "SM count");
+    // per-CTA moment accumulators in dynamic shared memory when they fit without costing residency
+    const size_t mom_bytes = (size_t)T * (1 + 3 * (size_t)S) * 8;
     int occ = 0;
     ckd(d.Occupancy(&occ, m->function, m->block_threads, 0), "occupancy");
     if (occ < 1) fail(CWC_E_CUDA, "kernel cannot be resident with block_threads = " + std::to_string(m->block_threads));
+    size_t dyn_smem = 0;
+    if (m->smem_stats && mom_bytes <= (size_t)200 * 1024) {
+        ckd(d.FuncSetAttribute(m->function, CU_FUNC_ATTRIBUTE_MAX_DYNAMIC_SHARED_SIZE_BYTES, (int)mom_bytes),
+            "dynamic smem");
+        int occ2 = 0;
+        ckd(d.Occupancy(&occ2, m->function, m->block_threads, mom_bytes), "occupancy");
+        if (occ2 >= occ) dyn_smem = mom_bytes;
+    }
     int per_sm = m->blocks_per_sm > 0 ? std::min(m->blocks_per_sm, occ) : occ;
     int64_t grid = (int64_t)sms * per_sm;
     // Every resident slot is launched even when there are fewer instances than lanes: warps race
@@ -453,13 +465,15 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     P.st_qdone = (unsigned int*)(sc + L.qdone);
     P.work = (unsigned long long*)(sc + L.work);
     P.logtab = m->d_logtab;
+    P.smem_stats = dyn_smem ? 1 : 0;
 
     ck(cudaMemsetAsync(m->d_stats, 0, need_stats * 8, stream), "memset(stats)");
     ck(cudaMemsetAsync(sc + L.qdone, 0, L.work + 8 - L.qdone, stream), "memset(queue)");
     ck(cudaEventRecord(m->ev0, stream), "cudaEventRecord");
     if (count > 0) {
         void* args[] = {&P};
-        ckd(d.LaunchKernel(m->function, (unsigned)grid, 1, 1, (unsigned)m->block_threads, 1, 1, 0, (CUstream)stream,
+        ckd(d.LaunchKernel(m->function, (unsigned)grid, 1, 1, (unsigned)m->block_threads, 1, 1, (unsigned)dyn_smem,
+                           (CUstream)stream,
                            args, nullptr),
             "cuLaunchKernel");
     }

@@ -24,6 +24,7 @@ struct cwc_model {
     int block_threads = 256;
     int min_blocks = 0;
     int ilp = 1;
+    int smem_stats = 1;
     int blocks_per_sm = 0;
     int refill = 1;
     int device = -1;
