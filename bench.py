@@ -194,9 +194,15 @@ def run_b200(args):
         if world == 1 and args.gpus > 1:
             print(f"--gpus {args.gpus} needs torchrun with {args.gpus} processes", file=sys.stderr)
             return 2
+    # one process per GPU; CWC_DIST_BACKEND=gloo lets a functional multi-rank run share one GPU
+    backend = os.environ.get("CWC_DIST_BACKEND", "nccl")
+    local = local % max(1, torch.cuda.device_count()) if backend != "nccl" else local
     torch.cuda.set_device(local)
     if world > 1:
-        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+        if backend == "nccl":
+            dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+        else:
+            dist.init_process_group(backend)
     cfg = W.CONFIGS[args.config]
     n_per = args.instances or cfg.n_instances
     n_total = n_per * world
@@ -213,7 +219,10 @@ def run_b200(args):
 
     def barrier():
         if world > 1:
-            dist.barrier(device_ids=[local])
+            if backend == "nccl":
+                dist.barrier(device_ids=[local])
+            else:
+                dist.barrier()
 
     for w in range(args.warmup):
         with torch.cuda.stream(stream):
