@@ -227,6 +227,8 @@ cwc_status cwc_instance_records(cwc_model_t m, int64_t first, int64_t count, uin
 cwc_status cwc_selftest_philox(int64_t n, const uint32_t* ctr, const uint32_t* key, uint32_t* out);
 cwc_status cwc_selftest_log(int64_t n, const double* x, double* out);
 cwc_status cwc_selftest_u01(int64_t n, const uint32_t* words, double* out); /* words [n][2] */
+/* The SSA kernel's branch-free IEEE division (round to nearest) for n pairs, host in/out. */
+cwc_status cwc_selftest_div(int64_t n, const double* num, const double* den, double* out);
 
 /* Library version string. */
 const char* cwc_version(void);

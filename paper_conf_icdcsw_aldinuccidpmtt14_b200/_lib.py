@@ -70,13 +70,14 @@ SIGNATURES = {
     "cwc_selftest_philox": (c_i32, [c_i64, c_vp, c_vp, c_vp]),
     "cwc_selftest_log": (c_i32, [c_i64, c_vp, c_vp]),
     "cwc_selftest_u01": (c_i32, [c_i64, c_vp, c_vp]),
+    "cwc_selftest_div": (c_i32, [c_i64, c_vp, c_vp, c_vp]),
 }
 
 
 def _load():
     if not os.path.exists(SO_PATH):
-        raise ImportError(f"{SO_PATH} is missing: build it with `python -m "
-                          f"paper_conf_icdcsw_aldinuccidpmtt14_b200.build` (there is no fallback)")
+        raise ImportError(f"{SO_PATH} is missing: build it with `python "
+                          f"paper_conf_icdcsw_aldinuccidpmtt14_b200/build.py` (there is no fallback)")
     lib = ctypes.CDLL(SO_PATH)
     for name, (res, args) in SIGNATURES.items():
         fn = getattr(lib, name)

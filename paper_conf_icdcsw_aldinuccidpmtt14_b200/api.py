@@ -281,3 +281,12 @@ def selftest_u01(words: np.ndarray) -> np.ndarray:
     out = np.empty(len(w), dtype=np.float64)
     check(lib.cwc_selftest_u01(len(w), _ptr(w), _ptr(out)))
     return out
+
+
+def selftest_div(num: np.ndarray, den: np.ndarray) -> np.ndarray:
+    """The SSA kernel's branch-free IEEE division, evaluated on the GPU."""
+    a = np.ascontiguousarray(num, dtype=np.float64)
+    b = np.ascontiguousarray(den, dtype=np.float64)
+    out = np.empty_like(a)
+    check(lib.cwc_selftest_div(len(a), _ptr(a), _ptr(b), _ptr(out)))
+    return out

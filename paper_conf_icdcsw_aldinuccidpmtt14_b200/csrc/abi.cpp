@@ -335,6 +335,13 @@ cwc_status cwc_selftest_log(int64_t n, const double* x, double* out) {
     });
 }
 
+cwc_status cwc_selftest_div(int64_t n, const double* num, const double* den, double* out) {
+    return guard([&] {
+        need(n >= 0 && (n == 0 || (num && den && out)), "bad arguments");
+        cwc::selftest_div(n, num, den, out);
+    });
+}
+
 cwc_status cwc_selftest_u01(int64_t n, const uint32_t* w, double* out) {
     return guard([&] {
         need(n >= 0 && (n == 0 || (w && out)), "bad arguments");

@@ -92,6 +92,7 @@ int64_t grid_K(double t_end, double dt);  // R13, throws CWC_E_INVALID
 void selftest_philox(int64_t n, const uint32_t* ctr, const uint32_t* key, uint32_t* out);
 void selftest_log(int64_t n, const double* x, double* out);
 void selftest_u01(int64_t n, const uint32_t* words, double* out);
+void selftest_div(int64_t n, const double* num, const double* den, double* out);
 void build_log_table(cwc_logtab_entry* tab);
 
 }  // namespace cwc

@@ -46,6 +46,11 @@ __global__ void k_u01(int64_t n, const uint32_t* w, double* out) {
     if (i < n) out[i] = cwc_u01(w[2 * i], w[2 * i + 1], s.k[6]);
 }
 
+__global__ void k_div(int64_t n, const double* num, const double* den, double* out) {
+    int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
+    if (i < n) out[i] = cwc_div(num[i], den[i]);
+}
+
 void ck(cudaError_t e, const char* what) {
     if (e != cudaSuccess) throw cwc::Error(CWC_E_CUDA, std::string(what) + ": " + cudaGetErrorString(e));
 }
@@ -81,6 +86,15 @@ void selftest_log(int64_t n, const double* x, double* out) {
     ck(cudaGetLastError(), "k_log");
     ck(cudaMemcpy(out, dout, n * sizeof(double), cudaMemcpyDeviceToHost), "D2H");
     cudaFree(dt); cudaFree(dx); cudaFree(dout);
+}
+
+void selftest_div(int64_t n, const double* num, const double* den, double* out) {
+    if (n <= 0) return;
+    double *dn = dev_copy(num, n), *dd = dev_copy(den, n), *dout = dev_copy<double>(nullptr, n);
+    k_div<<<(unsigned)((n + 255) / 256), 256>>>(n, dn, dd, dout);
+    ck(cudaGetLastError(), "k_div");
+    ck(cudaMemcpy(out, dout, n * sizeof(double), cudaMemcpyDeviceToHost), "D2H");
+    cudaFree(dn); cudaFree(dd); cudaFree(dout);
 }
 
 void selftest_u01(int64_t n, const uint32_t* words, double* out) {

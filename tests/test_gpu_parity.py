@@ -178,3 +178,20 @@ def test_full_size_sampled(cname):
         assert np.array_equal(raw[:, :, i], o.raw[:, :, 0]), i
         assert reactions[i] == o.reactions[0] and flags[i] == o.flags[0]
     assert res.reactions == int(reactions.sum())
+
+
+def test_device_fast_division_is_ieee():
+    """The kernel's branch-free divide (tau = -log(u) / a0) equals IEEE division bit for bit."""
+    from paper_conf_icdcsw_aldinuccidpmtt14_b200.api import selftest_div
+    rng = np.random.default_rng(4)
+    n = 4_000_000
+    num = -np.log(rng.random(n))                       # the SSA's numerators: -log(u), u in (0,1)
+    num[:1000] = np.exp2(-rng.random(1000) * 53)       # tiny -log(u)
+    den = np.exp2(rng.uniform(-60, 60, n)) * rng.uniform(1, 2, n)   # propensity sums over 36 decades
+    den[:500] = 1.0
+    den[500:1000] = np.round(rng.uniform(1, 1e6, 500))   # exact-quotient / integer cases
+    num[500:1000] = den[500:1000] * np.round(rng.uniform(1, 30, 500))
+    den[1000:1100] = 2.0 ** rng.integers(-1100, 1100, 100)  # out of the fast range -> fallback
+    got = selftest_div(num, den)
+    ref = num / den
+    assert np.array_equal(got.view(np.uint64), ref.view(np.uint64))
