@@ -181,6 +181,10 @@ cwc_status cwc_simulate_range(cwc_model_t m, int64_t n_total, int64_t first, int
 #define CWC_CTR_OVERFLOWED 2
 #define CWC_CTR_FINISHED 3
 #define CWC_N_CTR 8
+/* With period analysis on ("period_species" >= 0), CWC_N_PERIOD arrays of T int64 follow the
+ * counters: events, completed periods n / sum / sq_lo / sq_hi, local period n / sum / sq_lo /
+ * sq_hi (periods in cuts; sq split like sqlo/sqhi). */
+#define CWC_N_PERIOD 9
 cwc_status cwc_stats_device(cwc_model_t m, int64_t** dptr, size_t* n_int64);
 
 /* Synchronise, copy the packed stats to the host and derive mean, variance (n-1; int128
@@ -210,6 +214,31 @@ typedef struct {
 } cwc_stats_t;
 /* Borrowed views into the handle, valid until the next simulate / finalize / free. */
 cwc_status cwc_stats(cwc_model_t m, cwc_stats_t* out);
+
+/* ------------------------------------------------------------------------------------------
+ * On-line oscillation-period analysis ("we compute the
+ * period of each oscillation and plot the moving average ... of the local period", on sliding
+ * windows over the cuts P:L252-258).  Enabled per model with the options
+ *   "period_species" (flat index, -1 = off) or "period_species.<name>" = 1,
+ *   "period_lo" < "period_hi" (Schmitt-trigger thresholds on the species count),
+ *   "period_window" (moving-average window in cuts, default 1).
+ * Reading R19: an instance's detector is armed by a cut with x <= lo and fires an
+ * event at the first later cut with x >= hi; a period is the number of cuts between consecutive
+ * events; the local period of an instance at cut k is its last completed period.  All counts
+ * are exact integers accumulated by the SSA kernel (same packed buffer, all-reduce-summable).
+ * Views are valid until the next simulate / finalize / free; CWC_E_STATE if the analysis was off. */
+typedef struct {
+    int32_t T, species, window;
+    int64_t lo, hi;
+    const int64_t* events;                            /* [T] events at cut k */
+    const int64_t *pc_n, *pc_sum, *pc_sqlo, *pc_sqhi; /* [T] periods (in cuts) completing at k */
+    const int64_t *lp_n, *lp_sum, *lp_sqlo, *lp_sqhi; /* [T] local periods of instances at k */
+    const double* lp_mean;                            /* [T] mean local period, time units */
+    const double* lp_var;                             /* [T] its unbiased variance, time^2 */
+    const double* moving_avg;                         /* [T] mean of periods completed in the
+                                                         `window` cuts ending at k, time units */
+} cwc_period_stats_t;
+cwc_status cwc_period_stats(cwc_model_t m, cwc_period_stats_t* out);
 
 /* Raw samples of local instances [first, first+count) of the last simulated range, copied to
  * host out[T][S][count] (-1 = missing after an overflow).  CWC_E_STATE if raw_samples = 0. */

@@ -88,10 +88,17 @@ def period_stats(raw: np.ndarray, species: int, lo: int, hi: int) -> PeriodStats
 
 
 def finalize(ps: PeriodStats, dt: float, window: int):
-    """Mean local period per cut and the W-cut moving average of completed periods (time units)."""
+    """Mean local period per cut, the W-cut moving average of completed periods (time units) and
+    the unbiased variance of the local period (time^2): (mean, moving average, variance)."""
     T = len(ps.ev)
     lp_mean = np.array([float(int(ps.lp_sum[k])) / float(int(ps.lp_n[k])) * dt if ps.lp_n[k] else np.nan
                         for k in range(T)])
+    lp_var = np.full(T, np.nan)
+    for k in range(T):
+        n = int(ps.lp_n[k])
+        if n > 1:
+            s, q = int(ps.lp_sum[k]), int(ps.lp_sq[k])
+            lp_var[k] = float(n * q - s * s) / float(n * (n - 1)) * dt * dt
     ma = np.full(T, np.nan)
     for k in range(T):
         a = max(0, k - window + 1)
@@ -99,4 +106,4 @@ def finalize(ps: PeriodStats, dt: float, window: int):
         s = int(ps.pc_sum[a:k + 1].sum())
         if n:
             ma[k] = float(s) / float(n) * dt
-    return lp_mean, ma
+    return lp_mean, ma, lp_var

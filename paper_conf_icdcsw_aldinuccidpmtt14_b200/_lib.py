@@ -47,6 +47,13 @@ class Stats(ctypes.Structure):
                 ("finished", c_i64), ("kernel_ms", c_dbl), ("species_names", P(c_cp))]
 
 
+class PeriodStats(ctypes.Structure):
+    _fields_ = [("T", c_i32), ("species", c_i32), ("window", c_i32), ("lo", c_i64), ("hi", c_i64),
+                ("events", P(c_i64)), ("pc_n", P(c_i64)), ("pc_sum", P(c_i64)), ("pc_sqlo", P(c_i64)),
+                ("pc_sqhi", P(c_i64)), ("lp_n", P(c_i64)), ("lp_sum", P(c_i64)), ("lp_sqlo", P(c_i64)),
+                ("lp_sqhi", P(c_i64)), ("lp_mean", P(c_dbl)), ("lp_var", P(c_dbl)), ("moving_avg", P(c_dbl))]
+
+
 # name -> (restype, argtypes)
 SIGNATURES = {
     "cwc_version": (c_cp, []),
@@ -66,6 +73,7 @@ SIGNATURES = {
     "cwc_stats_finalize": (c_i32, [c_vp, c_vp]),
     "cwc_stats": (c_i32, [c_vp, P(Stats)]),
     "cwc_samples": (c_i32, [c_vp, c_i64, c_i64, c_vp]),
+    "cwc_period_stats": (c_i32, [c_vp, P(PeriodStats)]),
     "cwc_instance_records": (c_i32, [c_vp, c_i64, c_i64, c_vp, c_vp, c_vp]),
     "cwc_selftest_philox": (c_i32, [c_i64, c_vp, c_vp, c_vp]),
     "cwc_selftest_log": (c_i32, [c_i64, c_vp, c_vp]),

@@ -63,7 +63,8 @@ class Model:
                  *, x_cap: Optional[int] = None, hist_bins: Optional[int] = None, hist_width=None, hist_lo=None,
                  quantiles: Optional[Sequence[float]] = None, raw_samples: bool = True,
                  quantum_samples: int = 0, block_threads: Optional[int] = None, refill: bool = True,
-                 blocks_per_sm: int = 0, device: Optional[int] = None, **options):
+                 blocks_per_sm: int = 0, device: Optional[int] = None, period_species=None,
+                 period_lo: int = 0, period_hi: int = 1, period_window: int = 1, **options):
         sp = (ctypes.c_char_p * len(species))(*[s.encode() for s in species])
         rl = (ctypes.c_char_p * max(len(rules), 1))(*[r.encode() for r in rules])
         rt = (ctypes.c_double * max(len(rates), 1))(*[float(k) for k in rates])
@@ -93,6 +94,14 @@ class Model:
         self.set_option("blocks_per_sm", int(blocks_per_sm))
         for key, val in options.items():
             self.set_option(key, int(val))
+        if period_species is not None:   # on-line oscillation-period analysis (R19)
+            if isinstance(period_species, str):
+                self.set_option(f"period_species.{period_species}", 1)
+            else:
+                self.set_option("period_species", int(period_species))
+            self.set_option("period_lo", int(period_lo))
+            self.set_option("period_hi", int(period_hi))
+            self.set_option("period_window", int(period_window))
         if device is not None:
             self.set_option("device", int(device))
 
@@ -213,6 +222,18 @@ class Model:
             reactions=st.reactions, absorbed=st.absorbed, overflowed=st.overflowed, finished=st.finished,
             kernel_ms=st.kernel_ms, species=[st.species_names[s].decode() for s in range(S)],
         )
+
+    def period_stats(self) -> dict:
+        """On-line period analysis of the last simulation (cwc_period_stats) as numpy arrays."""
+        ps = _lib.PeriodStats()
+        check(lib.cwc_period_stats(self._h, ctypes.byref(ps)))
+        T = ps.T
+        out = dict(species=ps.species, window=ps.window, lo=ps.lo, hi=ps.hi)
+        for name in ("events", "pc_n", "pc_sum", "pc_sqlo", "pc_sqhi", "lp_n", "lp_sum", "lp_sqlo", "lp_sqhi"):
+            out[name] = np.ctypeslib.as_array(getattr(ps, name), shape=(T,)).astype(np.int64, copy=True)
+        for name in ("lp_mean", "lp_var", "moving_avg"):
+            out[name] = np.ctypeslib.as_array(getattr(ps, name), shape=(T,)).astype(np.float64, copy=True)
+        return out
 
     def stats_device(self):
         p, n = ctypes.c_void_p(), ctypes.c_size_t()

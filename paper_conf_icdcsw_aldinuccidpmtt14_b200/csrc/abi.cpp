@@ -168,6 +168,23 @@ cwc_status cwc_set_option_i64(cwc_model_t m, const char* key, int64_t v) {
         } else if (k == "block_threads") {
             need(v >= 32 && v <= 1024 && v % 32 == 0, "block_threads: multiple of 32 in [32, 1024]");
             m->block_threads = (int)v;
+        } else if (k == "period_species") {
+            need(v >= -1 && v < m->fm.S(), "period_species: flat species index or -1");
+            m->period_species = (int)v;
+        } else if (k.rfind("period_species.", 0) == 0) {
+            need(v == 0 || v == 1, "period_species.<name> is 0 or 1");
+            const int s = species_index(m, k.substr(15));
+            if (v) m->period_species = s;
+            else if (m->period_species == s) m->period_species = -1;
+        } else if (k == "period_lo") {
+            need(std::llabs(v) <= (int64_t)1 << 40, "period_lo out of range");
+            m->period_lo = v;
+        } else if (k == "period_hi") {
+            need(std::llabs(v) <= (int64_t)1 << 40, "period_hi out of range");
+            m->period_hi = v;
+        } else if (k == "period_window") {
+            need(v >= 1 && v <= (int64_t)1 << 30, "period_window >= 1");
+            m->period_window = (int)v;
         } else if (k == "smem_stats") {
             need(v == 0 || v == 1, "smem_stats is 0 or 1");
             m->smem_stats = (int)v;
@@ -303,6 +320,34 @@ cwc_status cwc_stats(cwc_model_t m, cwc_stats_t* out) {
         out->finished = ctr[CWC_CTR_FINISHED];
         out->kernel_ms = m->kernel_ms;
         out->species_names = m->name_ptrs.data();
+    });
+}
+
+cwc_status cwc_period_stats(cwc_model_t m, cwc_period_stats_t* out) {
+    return guard([&] {
+        need(m && out, "NULL argument");
+        if (!m->finalized) fail(CWC_E_STATE, "call cwc_stats_finalize after simulating");
+        if (m->h_period.empty()) fail(CWC_E_STATE, "period analysis was off for the last simulation");
+        const int64_t T = m->K + 1;
+        const int64_t* q = m->h_period.data();
+        std::memset(out, 0, sizeof *out);
+        out->T = (int32_t)T;
+        out->species = m->period_species;
+        out->window = m->period_window;
+        out->lo = m->period_lo;
+        out->hi = m->period_hi;
+        out->events = q;
+        out->pc_n = q + T;
+        out->pc_sum = q + 2 * T;
+        out->pc_sqlo = q + 3 * T;
+        out->pc_sqhi = q + 4 * T;
+        out->lp_n = q + 5 * T;
+        out->lp_sum = q + 6 * T;
+        out->lp_sqlo = q + 7 * T;
+        out->lp_sqhi = q + 8 * T;
+        out->lp_mean = m->lp_mean.data();
+        out->lp_var = m->lp_var.data();
+        out->moving_avg = m->p_ma.data();
     });
 }
 

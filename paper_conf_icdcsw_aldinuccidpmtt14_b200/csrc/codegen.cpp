@@ -27,6 +27,8 @@ std::string generate_model_section(const FlatModel& fm, const KernelConfig& cfg)
     o << "// ---- generated model section: " << S << " species, " << M << " flat reactions\n";
     o << "#define CWC_S " << S << "\n#define CWC_M " << (M > 0 ? M : 1) << "\n#define CWC_B " << cfg.hist_bins
       << "\n#define CWC_BLOCK " << cfg.block_threads << "\n#define CWC_MINB " << cfg.min_blocks << "\n#define CWC_ILP " << cfg.ilp << "\n";
+    o << "#define CWC_PERIOD_S " << cfg.period_species << "\n#define CWC_PERIOD_LO " << cfg.period_lo
+      << "LL\n#define CWC_PERIOD_HI " << cfg.period_hi << "LL\n";
     o << "#define CWC_X_CAP " << cfg.x_cap << "\n\n";
     if (cfg.seed_keys) {
         const uint32_t k0 = (uint32_t)cfg.seed, k1 = (uint32_t)(cfg.seed >> 32);

@@ -15,6 +15,8 @@ struct KernelConfig {
     int hist_bins = 256;
     bool seed_keys = false;  // bake the Philox round keys of `seed` into the kernel (immediates)
     uint64_t seed = 0;
+    int period_species = -1;  // on-line period detector on this flat species (-1 = off)
+    int64_t period_lo = 0, period_hi = 1;
     int64_t x_cap = 0;
     std::vector<int64_t> hist_lo, hist_width;  // [S]
 };

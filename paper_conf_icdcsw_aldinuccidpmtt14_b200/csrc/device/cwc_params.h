@@ -29,6 +29,7 @@ struct cwc_params {
     unsigned long long* st_step;  // [count] saved step (= reactions applied)
     long long* st_k;            // [count] next cut index
     unsigned int* st_flags;     // [count] CWC_FLAG_* | CWC_TERMINAL
+    unsigned long long* st_pd;  // [count] period-detector state (R19)
     unsigned int* st_qdone;     // [count] quanta completed (release/acquire)
     unsigned long long* work;   // work-queue counter
     const cwc_logtab_entry* logtab;  // [128]

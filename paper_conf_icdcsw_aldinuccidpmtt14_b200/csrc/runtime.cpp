@@ -89,18 +89,21 @@ int64_t grid_K(double t_end, double dt) {
     return K;
 }
 
-size_t stats_len(int64_t T, int S, int B) { return (size_t)(T * (1 + 3 * (int64_t)S + (int64_t)S * (B + 2)) + CWC_N_CTR); }
+size_t stats_len(int64_t T, int S, int B, bool period) {
+    return (size_t)(T * (1 + 3 * (int64_t)S + (int64_t)S * (B + 2)) + CWC_N_CTR + (period ? CWC_N_PERIOD * T : 0));
+}
 
 static size_t align256(size_t v) { return (v + 255) & ~(size_t)255; }
 
 struct ScratchLayout {
-    size_t x, t, step, k, flags, qdone, work, total;
+    size_t x, t, step, k, flags, pd, qdone, work, total;
 };
 
 static ScratchLayout scratch_layout(int S, int64_t count) {
     ScratchLayout L{};
     size_t off = 0;
     L.x = off; off = align256(off + (size_t)S * count * 4);
+    L.pd = off; off = align256(off + (size_t)count * 8);
     L.t = off; off = align256(off + (size_t)count * 8);
     L.step = off; off = align256(off + (size_t)count * 8);
     L.k = off; off = align256(off + (size_t)count * 8);
@@ -114,7 +117,7 @@ static ScratchLayout scratch_layout(int S, int64_t count) {
 
 void buffer_sizes(const cwc_model* m, int64_t count, int64_t K, size_t* stats, size_t* raw, size_t* scratch) {
     const int S = m->fm.S();
-    if (stats) *stats = stats_len(K + 1, S, m->hist_bins);
+    if (stats) *stats = stats_len(K + 1, S, m->hist_bins, m->period_species >= 0);
     if (raw) *raw = m->raw_samples ? (size_t)(K + 1) * S * (size_t)count : 0;
     if (scratch) *scratch = scratch_layout(S, count).total;
 }
@@ -218,6 +221,9 @@ void compile(cwc_model* m, const uint64_t* seed) {
     // App. B models (fewer, fatter threads lose more to latency than they gain from registers)
     cfg.min_blocks = m->min_blocks > 0 ? m->min_blocks : std::max(1, 768 / m->block_threads);
     cfg.ilp = m->ilp;
+    cfg.period_species = m->period_species;
+    cfg.period_lo = m->period_lo;
+    cfg.period_hi = m->period_hi;
     cfg.hist_bins = m->hist_bins;
     cfg.x_cap = m->x_cap;
     cfg.hist_lo = m->hist_lo;
@@ -374,6 +380,8 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     if (n_total <= 0) fail(CWC_E_INVALID, "n_total must be > 0");
     if (first < 0 || count < 0 || first + count > n_total) fail(CWC_E_INVALID, "instance range outside [0, n_total)");
     const int64_t K = grid_K(t_end, dt);
+    if (m->period_species >= 0 && !(m->period_lo < m->period_hi))
+        fail(CWC_E_INVALID, "period analysis needs period_lo < period_hi");
     const int64_t T = K + 1;
     const int S = m->fm.S();
     compile(m, &seed);
@@ -462,6 +470,7 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     P.st_step = (unsigned long long*)(sc + L.step);
     P.st_k = (long long*)(sc + L.k);
     P.st_flags = (unsigned int*)(sc + L.flags);
+    P.st_pd = (unsigned long long*)(sc + L.pd);
     P.st_qdone = (unsigned int*)(sc + L.qdone);
     P.work = (unsigned long long*)(sc + L.work);
     P.logtab = m->d_logtab;
@@ -532,6 +541,36 @@ void finalize(cwc_model* m, const int64_t* host_stats) {
     m->h_sqlo.assign(p + T + TS, p + T + 2 * TS);
     m->h_sqhi.assign(p + T + 2 * TS, p + T + 3 * TS);
     m->h_hist.assign(p + T + 3 * TS, p + T + 3 * TS + TS * (B + 2));
+    // on-line period analysis (R19): per-cut integers -> local-period mean / variance and the
+    // moving average of completed periods over the last `window` cuts, in time units
+    m->h_period.clear();
+    m->lp_mean.assign(T, NAN);
+    m->lp_var.assign(T, NAN);
+    m->p_ma.assign(T, NAN);
+    if (m->period_species >= 0) {
+        const int64_t* q = p + T + 3 * TS + TS * (B + 2) + CWC_N_CTR;
+        m->h_period.assign(q, q + CWC_N_PERIOD * T);
+        const int64_t *pcn = q + T, *pcs = q + 2 * T, *lpn = q + 5 * T, *lps = q + 6 * T;
+        const int64_t *lpl = q + 7 * T, *lph = q + 8 * T;
+        int64_t wn = 0, ws = 0;
+        for (int64_t k = 0; k < T; ++k) {
+            const int64_t n = lpn[k];
+            if (n > 0) m->lp_mean[k] = (double)lps[k] / (double)n * m->dt;
+            if (n > 1) {
+                const __int128 sq = ((__int128)(uint64_t)lph[k] << 32) + (__int128)(uint64_t)lpl[k];
+                const __int128 s = lps[k];
+                const double vc = (double)((__int128)n * sq - s * s) / (double)((__int128)n * (n - 1));
+                m->lp_var[k] = vc * m->dt * m->dt;
+            }
+            wn += pcn[k];
+            ws += pcs[k];
+            if (k >= m->period_window) {
+                wn -= pcn[k - m->period_window];
+                ws -= pcs[k - m->period_window];
+            }
+            if (wn > 0) m->p_ma[k] = (double)ws / (double)wn * m->dt;
+        }
+    }
     m->times.resize(T);
     m->mean.assign(TS, NAN);
     m->var.assign(TS, NAN);

@@ -25,6 +25,11 @@ struct cwc_model {
     int min_blocks = 0;
     int ilp = 1;
     int smem_stats = 1;
+    // on-line period analysis (reading R19): observable species (-1 = off), Schmitt thresholds,
+    // moving-average window in cuts
+    int period_species = -1;
+    int64_t period_lo = 0, period_hi = 1;
+    int period_window = 1;
     int blocks_per_sm = 0;
     int refill = 1;
     int device = -1;
@@ -70,6 +75,8 @@ struct cwc_model {
     std::vector<int64_t> h_stats;
     std::vector<double> times, mean, var, sumsq_d, quant;
     std::vector<int64_t> h_n, h_sum, h_sqlo, h_sqhi, h_hist;
+    std::vector<int64_t> h_period;             // CWC_N_PERIOD x T (R19)
+    std::vector<double> lp_mean, lp_var, p_ma;  // [T]
     double kernel_ms = 0;
 
     ~cwc_model();
@@ -77,7 +84,7 @@ struct cwc_model {
 
 namespace cwc {
 
-size_t stats_len(int64_t T, int S, int B);
+size_t stats_len(int64_t T, int S, int B, bool period);
 void buffer_sizes(const cwc_model* m, int64_t count, int64_t K, size_t* stats, size_t* raw, size_t* scratch);
 void compile(cwc_model* m, const uint64_t* seed = nullptr);  // NVRTC (no GPU needed)
 void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count, double t_end, double dt,

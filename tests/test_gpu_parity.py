@@ -195,3 +195,36 @@ def test_device_fast_division_is_ieee():
     got = selftest_div(num, den)
     ref = num / den
     assert np.array_equal(got.view(np.uint64), ref.view(np.uint64))
+
+
+# ------------------------------------------------------------------ on-line period analysis (R19)
+@pytest.mark.parametrize("md,species,lo,hi,t_end,dt,n", [
+    (W.CIRCADIAN, "R", 100, 1000, 96.0, 0.5, 1500),
+    (W.LOTKA_VOLTERRA, "Y1", 800, 1300, 10.0, 0.05, 1000),
+])
+def test_period_analysis_matches_oracle(md, species, lo, hi, t_end, dt, n):
+    from oracle.period import finalize, period_stats
+    import paper_conf_icdcsw_aldinuccidpmtt14_b200 as cwc
+    W_ = 24
+    m = cwc.Model.from_def(md, hist_bins=64, hist_width=64, period_species=species, period_lo=lo, period_hi=hi,
+                           period_window=W_)
+    seed = 2024
+    m.simulate_range(n, 0, n, t_end, dt, seed)
+    m.finalize()
+    got = m.period_stats()
+    fm = flatten_def(md)
+    orun = oracle.simulate(fm, 0, n, t_end, dt, seed, nthreads=16)
+    assert np.array_equal(m.samples(0, n), orun.raw)
+    ps = period_stats(orun.raw, fm.names.index(species), lo, hi)
+    assert got["species"] == fm.names.index(species)
+    assert np.array_equal(got["events"], ps.ev) and ps.ev.sum() > n
+    assert np.array_equal(got["pc_n"], ps.pc_n) and np.array_equal(got["pc_sum"], ps.pc_sum)
+    assert [(int(h) << 32) + int(l) for h, l in zip(got["pc_sqhi"], got["pc_sqlo"])] == list(ps.pc_sq)
+    assert np.array_equal(got["lp_n"], ps.lp_n) and np.array_equal(got["lp_sum"], ps.lp_sum)
+    assert [(int(h) << 32) + int(l) for h, l in zip(got["lp_sqhi"], got["lp_sqlo"])] == list(ps.lp_sq)
+    lp_mean, ma, lp_var = finalize(ps, dt, W_)
+    assert np.array_equal(got["lp_mean"], lp_mean, equal_nan=True)
+    assert np.array_equal(got["moving_avg"], ma, equal_nan=True)
+    assert np.array_equal(got["lp_var"], lp_var, equal_nan=True)
+    if md is W.CIRCADIAN:   # Vilar oscillator: local period ~ 20-30 h once every instance has one
+        assert 20.0 < np.nanmean(lp_mean[-48:]) < 30.0

@@ -34,7 +34,8 @@ def test_period_stats_and_moving_average():
     assert ps.lp_n.tolist() == [0, 0, 0, 0, 1, 1, 1, 1, 2, 2]
     assert ps.lp_sum.tolist() == [0, 0, 0, 0, 3, 3, 2, 2, 7, 7]
     assert list(ps.lp_sq) == [0, 0, 0, 0, 9, 9, 4, 4, 29, 29]
-    lp_mean, ma = finalize(ps, 0.5, window=3)
+    lp_mean, ma, lp_var = finalize(ps, 0.5, window=3)
+    assert lp_var[8] == (2 * 29 - 49) / 2 * 0.25 and np.isnan(lp_var[7])
     assert lp_mean[4] == 1.5 and lp_mean[9] == 3.5 * 0.5 and np.isnan(lp_mean[3])
     # window of 3 cuts ending at k: periods completing in [k-2, k]
     assert np.isnan(ma[3]) and ma[4] == 1.5 and ma[6] == (3 + 2) / 2 * 0.5 and ma[8] == (2 + 5) / 2 * 0.5
