@@ -191,7 +191,7 @@ def test_device_fast_division_is_ieee():
     den[:500] = 1.0
     den[500:1000] = np.round(rng.uniform(1, 1e6, 500))   # exact-quotient / integer cases
     num[500:1000] = den[500:1000] * np.round(rng.uniform(1, 30, 500))
-    den[1000:1100] = 2.0 ** rng.integers(-1100, 1100, 100)  # out of the fast range -> fallback
+    den[1000:1100] = np.ldexp(1.0, rng.integers(-1020, 1020, 100))  # out of the fast range -> fallback
     got = selftest_div(num, den)
     ref = num / den
     assert np.array_equal(got.view(np.uint64), ref.view(np.uint64))
