@@ -94,6 +94,13 @@ typedef struct {
     int32_t hist_bins;                /* B */
     const int64_t* hist_lo;           /* [n_species] */
     const int64_t* hist_width;        /* [n_species] */
+    /* functional rate laws (reading R16'; rule suffix "@ mm(X, K)", "@ hill(X, K, n)",
+     * "@ hillr(X, K, n)"): per flat reaction 0 mass action / 1 mm / 2 hill / 3 hillr, the
+     * flat species the law reads (-1 for mass action), K and n. */
+    const int32_t* law;
+    const int32_t* law_species;
+    const double* law_K;
+    const int32_t* law_n;
 } cwc_model_info_t;
 cwc_status cwc_model_info(cwc_model_t m, cwc_model_info_t* out);
 

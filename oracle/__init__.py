@@ -53,6 +53,10 @@ class _Model(ctypes.Structure):
         ("react_r", ctypes.POINTER(ctypes.c_int32)),
         ("delta", ctypes.POINTER(ctypes.c_int32)),
         ("x_cap", ctypes.c_int64),
+        ("law", ctypes.POINTER(ctypes.c_int32)),
+        ("law_s", ctypes.POINTER(ctypes.c_int32)),
+        ("law_K", ctypes.POINTER(ctypes.c_double)),
+        ("law_n", ctypes.POINTER(ctypes.c_int32)),
     ]
 
 
@@ -119,10 +123,17 @@ class CModel:
                 self.react_s[j * 4 + e] = s
                 self.react_r[j * 4 + e] = r
         self.delta = np.array(fm.delta, dtype=np.int32).reshape(-1) if M else np.zeros(1, np.int32)
+        nz = max(M, 1)
+        self.law = np.array(fm.law or [0] * nz, dtype=np.int32)
+        self.law_s = np.array(fm.law_species or [-1] * nz, dtype=np.int32)
+        self.law_K = np.array(fm.law_K or [0.0] * nz, dtype=np.float64)
+        self.law_n = np.array(fm.law_n or [1] * nz, dtype=np.int32)
         P = lambda a, t: a.ctypes.data_as(ctypes.POINTER(t))  # noqa: E731
         self.c = _Model(S, M, P(self.x0, ctypes.c_int32), P(self.k, ctypes.c_double),
                         P(self.n_react, ctypes.c_int32), P(self.react_s, ctypes.c_int32),
-                        P(self.react_r, ctypes.c_int32), P(self.delta, ctypes.c_int32), fm.x_cap)
+                        P(self.react_r, ctypes.c_int32), P(self.delta, ctypes.c_int32), fm.x_cap,
+                        P(self.law, ctypes.c_int32), P(self.law_s, ctypes.c_int32),
+                        P(self.law_K, ctypes.c_double), P(self.law_n, ctypes.c_int32))
 
     def propensities(self, x):
         x = np.ascontiguousarray(x, dtype=np.int32)

@@ -178,12 +178,49 @@ def parse_term(text: str, alphabet: Sequence[str]) -> Term:
     return Term(atoms, comps)
 
 
+LAW_MASS_ACTION, LAW_MM, LAW_HILL, LAW_HILLR = 0, 1, 2, 3
+_LAWS = {"mm": LAW_MM, "hill": LAW_HILL, "hillr": LAW_HILLR}
+
+
 @dataclass
 class Rule:
     label: str
     lhs: Pattern
     rhs: Pattern
     rate: float
+    law: int = LAW_MASS_ACTION   # reading R16': functional rate laws
+    law_atom: Optional[str] = None
+    law_K: float = 0.0
+    law_n: int = 1
+
+
+def parse_law(text: str, alphabet: Sequence[str]):
+    """'mm(X, K)' | 'hill(X, K, n)' | 'hillr(X, K, n)' -> (law, atom, K, n)."""
+    m = re.fullmatch(r"\s*(mm|hill|hillr)\s*\(\s*([A-Za-z_][A-Za-z0-9_]*)\s*,\s*([^,()]+?)\s*(?:,\s*([0-9]+)\s*)?\)\s*",
+                     text)
+    if not m:
+        raise CWCError("parse", f"bad rate law {text!r}")
+    law = _LAWS[m.group(1)]
+    atom = m.group(2)
+    if atom not in alphabet:
+        raise CWCError("invalid", f"unknown atom {atom!r} in rate law")
+    try:
+        K = float(m.group(3))
+    except ValueError:
+        raise CWCError("parse", f"bad constant in rate law {text!r}")
+    if not math.isfinite(K) or K <= 0:
+        raise CWCError("invalid", f"rate-law constant must be finite and > 0: {text!r}")
+    if law == LAW_MM:
+        if m.group(4) is not None:
+            raise CWCError("parse", f"mm takes (species, K): {text!r}")
+        n = 1
+    else:
+        if m.group(4) is None:
+            raise CWCError("parse", f"{m.group(1)} takes (species, K, n): {text!r}")
+        n = int(m.group(4))
+        if not 1 <= n <= 8:
+            raise CWCError("invalid", f"Hill exponent must be in [1, 8]: {text!r}")
+    return law, atom, K, n
 
 
 def parse_rule(text: str, alphabet: Sequence[str], rate: float) -> Rule:
@@ -193,6 +230,10 @@ def parse_rule(text: str, alphabet: Sequence[str], rate: float) -> Rule:
         raise CWCError("parse", f"rule without label: {text!r}")
     label, body = text.split(":", 1)
     label = label.strip()
+    law = (LAW_MASS_ACTION, None, 0.0, 1)
+    if "@" in body:
+        body, law_txt = body.split("@", 1)
+        law = parse_law(law_txt, alphabet)
     if not re.fullmatch(r"[A-Za-z_][A-Za-z0-9_]*", label):
         raise CWCError("parse", f"bad rule label {label!r}")
     if body.count("->") != 1:
@@ -224,7 +265,7 @@ def parse_rule(text: str, alphabet: Sequence[str], rate: float) -> Rule:
             if v in seen:
                 raise CWCError("unsupported", f"variable {v} used twice: {text!r}")
             seen.add(v)
-    return Rule(label, lhs, rhs, float(rate))
+    return Rule(label, lhs, rhs, float(rate), *law)
 
 
 # ------------------------------------------------------------------------------------------
@@ -278,6 +319,10 @@ class FlatModel:
     delta: List[List[int]]                   # per reaction: dense net change [S]
     rule_of: List[int]                       # originating CWC rule index
     x_cap: int
+    law: List[int] = field(default_factory=list)          # per reaction: LAW_* (R16')
+    law_species: List[int] = field(default_factory=list)  # species the law reads (-1: none)
+    law_K: List[float] = field(default_factory=list)
+    law_n: List[int] = field(default_factory=list)
 
 
 def _species_name(region: Region, atom: str) -> str:
@@ -353,7 +398,7 @@ def flatten(alphabet: Sequence[str], rules: Sequence[str], rates: Sequence[float
                     raise CWCError("unsupported", f"reaction order > 3 in rule {ri}")
                 delta = Counter(prod)
                 delta.subtract(react)
-                raw_reactions.append((ri, rule.rate, react, delta))
+                raw_reactions.append((ri, rule.rate, react, delta, ci))
 
     # --- species: referenced (region, atom) pairs, region pre-order then alphabet order -----
     used = set()
@@ -361,9 +406,11 @@ def flatten(alphabet: Sequence[str], rules: Sequence[str], rates: Sequence[float
         for atom, n in reg.atoms.items():
             if n > 0:
                 used.add((ri_, atom))
-    for _, _, react, delta in raw_reactions:
+    for ri, _, react, delta, ci in raw_reactions:
         used.update(react.keys())
         used.update(key for key, v in delta.items())
+        if parsed[ri].law != LAW_MASS_ACTION:
+            used.add((ci, parsed[ri].law_atom))
     aidx = {a: i for i, a in enumerate(alphabet)}
     species = sorted(used, key=lambda ra: (ra[0], aidx[ra[1]]))
     sidx = {sp: i for i, sp in enumerate(species)}
@@ -374,7 +421,13 @@ def flatten(alphabet: Sequence[str], rules: Sequence[str], rates: Sequence[float
     x0 = [regions[r].atoms.get(a, 0) for r, a in species]
 
     reactants, deltas, rates_f, rule_of = [], [], [], []
-    for ri, rate, react, delta in raw_reactions:
+    law, law_sp, law_K, law_n = [], [], [], []
+    for ri, rate, react, delta, ci in raw_reactions:
+        rl = parsed[ri]
+        law.append(rl.law)
+        law_sp.append(sidx[(ci, rl.law_atom)] if rl.law != LAW_MASS_ACTION else -1)
+        law_K.append(rl.law_K)
+        law_n.append(rl.law_n)
         reactants.append(sorted((sidx[sp], n) for sp, n in react.items() if n > 0))
         d = [0] * S
         for sp, n in delta.items():
@@ -390,7 +443,7 @@ def flatten(alphabet: Sequence[str], rules: Sequence[str], rates: Sequence[float
         raise CWCError("invalid", f"x_cap {x_cap} outside [1, {cap_max}]")
     if any(v > x_cap for v in x0):
         raise CWCError("invalid", "initial count above x_cap")
-    return FlatModel(species, names, x0, rates_f, reactants, deltas, rule_of, x_cap)
+    return FlatModel(species, names, x0, rates_f, reactants, deltas, rule_of, x_cap, law, law_sp, law_K, law_n)
 
 
 def flatten_def(model) -> FlatModel:

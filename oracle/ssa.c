@@ -144,6 +144,10 @@ typedef struct {
     const int32_t* react_r;  /* [M*4] reactant orders (stoichiometric coefficient) */
     const int32_t* delta;    /* [M*S] dense net change nu_j */
     int64_t x_cap;           /* reading R9 */
+    const int32_t* law;      /* [M] 0 mass action, 1 mm, 2 hill, 3 hillr (reading R16') */
+    const int32_t* law_s;    /* [M] species the law reads */
+    const double* law_K;     /* [M] */
+    const int32_t* law_n;    /* [M] Hill exponent */
 } oracle_model;
 
 enum { ORACLE_FLAG_ABSORBED = 1, ORACLE_FLAG_OVERFLOWED = 2 };
@@ -155,6 +159,29 @@ static uint64_t binom(int64_t x, int r) {
     uint64_t c = 1;
     for (int i = 0; i < r; ++i) c = c * (uint64_t)(x - i) / (uint64_t)(i + 1);
     return c;
+}
+
+/* a_j of one flat reaction.  Mass action (R1): fl(k_j * h_j).  Functional rate laws (reading
+ * R16') apply only when the lhs is available (h_j > 0); with X = (double)x_s of
+ * the law's species and Y^n = fl(...fl(fl(Y*Y)*Y)...) (n-1 left-to-right products):
+ *   mm:    fl(fl(k*X) / fl(K + X))            Michaelis-Menten
+ *   hill:  fl(fl(k*X^n) / fl(K^n + X^n))      Hill activation
+ *   hillr: fl(fl(k*K^n) / fl(K^n + X^n))      Hill repression */
+static double ipow(double y, int n) {
+    double r = y;
+    for (int i = 1; i < n; ++i) r = r * y;
+    return r;
+}
+
+static double propensity(const oracle_model* m, int32_t j, const int32_t* x, uint64_t h) {
+    const int law = m->law ? m->law[j] : 0;
+    if (law == 0) return m->k[j] * (double)h;
+    if (h == 0) return 0.0;
+    const double X = (double)x[m->law_s[j]], K = m->law_K[j];
+    if (law == 1) return (m->k[j] * X) / (K + X);
+    const double Xn = ipow(X, m->law_n[j]), Kn = ipow(K, m->law_n[j]);
+    if (law == 2) return (m->k[j] * Xn) / (Kn + Xn);
+    return (m->k[j] * Kn) / (Kn + Xn);
 }
 
 typedef struct {
@@ -201,7 +228,7 @@ static void simulate_instance(const job_t* jb, int64_t li) {
             uint64_t h = 1;
             for (int32_t e = 0; e < m->n_react[j]; ++e)
                 h *= binom(x[m->react_s[j * 4 + e]], m->react_r[j * 4 + e]);
-            a[j] = m->k[j] * (double)h;
+            a[j] = propensity(m, j, x, h);
         }
         /* a0 as a left-to-right running sum (R5) */
         double c = 0.0;
@@ -280,7 +307,7 @@ void oracle_propensities(const oracle_model* m, const int32_t* x, double* a, dou
         uint64_t h = 1;
         for (int32_t e = 0; e < m->n_react[j]; ++e)
             h *= binom(x[m->react_s[j * 4 + e]], m->react_r[j * 4 + e]);
-        a[j] = m->k[j] * (double)h;
+        a[j] = propensity(m, j, x, h);
         c = c + a[j];
         cum[j] = c;
     }

@@ -35,7 +35,8 @@ class ModelInfo(ctypes.Structure):
                 ("species_names", P(c_cp)), ("x0", P(c_i32)), ("rates", P(c_dbl)),
                 ("n_reactants", P(c_i32)), ("reactant_species", P(c_i32)), ("reactant_order", P(c_i32)),
                 ("delta", P(c_i32)), ("rule_of", P(c_i32)), ("x_cap", c_i64), ("x_cap_max", c_i64),
-                ("hist_bins", c_i32), ("hist_lo", P(c_i64)), ("hist_width", P(c_i64))]
+                ("hist_bins", c_i32), ("hist_lo", P(c_i64)), ("hist_width", P(c_i64)),
+                ("law", P(c_i32)), ("law_species", P(c_i32)), ("law_K", P(c_dbl)), ("law_n", P(c_i32))]
 
 
 class Stats(ctypes.Structure):

@@ -152,6 +152,8 @@ class Model:
                 rule_of=[mi.rule_of[j] for j in range(M)],
                 x_cap=mi.x_cap, x_cap_max=mi.x_cap_max, n_rules=mi.n_rules, hist_bins=mi.hist_bins,
                 hist_lo=[mi.hist_lo[s] for s in range(S)], hist_width=[mi.hist_width[s] for s in range(S)],
+                law=[mi.law[j] for j in range(M)], law_species=[mi.law_species[j] for j in range(M)],
+                law_K=[mi.law_K[j] for j in range(M)], law_n=[mi.law_n[j] for j in range(M)],
             )
         return self._info_cache
 

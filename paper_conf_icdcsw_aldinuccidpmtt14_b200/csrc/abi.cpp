@@ -133,6 +133,10 @@ cwc_status cwc_model_info(cwc_model_t m, cwc_model_info_t* out) {
         out->hist_bins = m->hist_bins;
         out->hist_lo = m->hist_lo.data();
         out->hist_width = m->hist_width.data();
+        out->law = m->fm.law.data();
+        out->law_species = m->fm.law_species.data();
+        out->law_K = m->fm.law_K.data();
+        out->law_n = m->fm.law_n.data();
     });
 }
 

@@ -55,8 +55,10 @@ std::string generate_model_section(const FlatModel& fm, const KernelConfig& cfg)
         o << "__device__ __forceinline__ int cwc_last_positive(const int (&x)[CWC_S]) {\n    double a[CWC_M];\n";
     // per-(species, order) binomial factors, shared between reactions
     std::vector<std::vector<bool>> need(S, std::vector<bool>(4, false));
-    for (int j = 0; j < M; ++j)
+    for (int j = 0; j < M; ++j) {
         for (const Reactant& r : fm.reactants[j]) need[r.species][r.order] = true;
+        if (fm.law[j] != LAW_MASS_ACTION) need[fm.law_species[j]][1] = true;
+    }
     for (int s = 0; s < S; ++s) {
         if (need[s][1] || need[s][2]) o << "    const double f" << s << "_1 = (double)x[" << s << "];\n";
         if (need[s][2])
@@ -73,8 +75,30 @@ std::string generate_model_section(const FlatModel& fm, const KernelConfig& cfg)
             std::string f = "f" + std::to_string(r.species) + "_" + std::to_string(r.order);
             h = h.empty() ? f : "__dmul_rn(" + h + ", " + f + ")";
         }
-        o << "    a[" << j << "] = " << (h.empty() ? hexd(fm.rates[j]) : "__dmul_rn(" + hexd(fm.rates[j]) + ", " + h + ")")
-          << ";  // rule " << fm.rule_of[j] << "\n";
+        if (fm.law[j] == LAW_MASS_ACTION) {
+            o << "    a[" << j << "] = "
+              << (h.empty() ? hexd(fm.rates[j]) : "__dmul_rn(" + hexd(fm.rates[j]) + ", " + h + ")")
+              << ";  // rule " << fm.rule_of[j] << "\n";
+            continue;
+        }
+        // functional rate law (R16'): k*X/(K+X), k*X^n/(K^n+X^n) or k*K^n/(K^n+X^n), only when the
+        // lhs is available; powers are left-to-right products, K^n computed on the host the same way
+        const std::string X = "f" + std::to_string(fm.law_species[j]) + "_1";
+        std::string Xn = X;
+        for (int i = 1; i < fm.law_n[j]; ++i) Xn = "__dmul_rn(" + Xn + ", " + X + ")";
+        double Kn = fm.law_K[j];
+        for (int i = 1; i < fm.law_n[j]; ++i) Kn = Kn * fm.law_K[j];
+        std::string expr;
+        if (fm.law[j] == LAW_MM)
+            expr = "cwc_div(__dmul_rn(" + hexd(fm.rates[j]) + ", " + X + "), __dadd_rn(" + hexd(fm.law_K[j]) + ", " +
+                   X + "))";
+        else if (fm.law[j] == LAW_HILL)
+            expr = "cwc_div(__dmul_rn(" + hexd(fm.rates[j]) + ", " + Xn + "), __dadd_rn(" + hexd(Kn) + ", " + Xn + "))";
+        else
+            expr = "cwc_div(__dmul_rn(" + hexd(fm.rates[j]) + ", " + hexd(Kn) + "), __dadd_rn(" + hexd(Kn) + ", " + Xn +
+                   "))";
+        o << "    a[" << j << "] = " << (h.empty() ? expr : "(" + h + " != 0.0) ? " + expr + " : 0.0")
+          << ";  // rule " << fm.rule_of[j] << " (rate law)\n";
     }
     if (variant == 0) {
         o << "    cum[0] = a[0];\n";

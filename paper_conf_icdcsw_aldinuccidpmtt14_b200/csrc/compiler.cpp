@@ -186,6 +186,10 @@ struct Rule {
     std::string label;
     Pattern lhs, rhs;
     double rate;
+    int32_t law = LAW_MASS_ACTION;  // "@ mm(X, K)" / "@ hill(X, K, n)" / "@ hillr(X, K, n)"
+    int law_atom = -1;
+    double law_K = 0.0;
+    int32_t law_n = 1;
 };
 
 bool valid_ident(const std::string& s) {
@@ -202,6 +206,43 @@ std::string trim(const std::string& s) {
     return s.substr(a, b - a);
 }
 
+// Rate-law suffix of a rule (reading R16'): "mm(X, K)" | "hill(X, K, n)" | "hillr(X, K, n)".
+void parse_law(const std::string& text, const std::unordered_map<std::string, int>& atoms, Rule& r) {
+    std::string t = trim(text);
+    size_t lp = t.find('('), rp = t.rfind(')');
+    if (lp == std::string::npos || rp == std::string::npos || rp < lp || trim(t.substr(rp + 1)) != "")
+        throw Error(CWC_E_PARSE, "bad rate law '" + t + "'");
+    const std::string name = trim(t.substr(0, lp));
+    std::vector<std::string> args;
+    std::string cur;
+    for (char c : t.substr(lp + 1, rp - lp - 1)) {
+        if (c == ',') { args.push_back(trim(cur)); cur.clear(); }
+        else cur += c;
+    }
+    args.push_back(trim(cur));
+    if (name == "mm") r.law = LAW_MM;
+    else if (name == "hill") r.law = LAW_HILL;
+    else if (name == "hillr") r.law = LAW_HILLR;
+    else throw Error(CWC_E_PARSE, "unknown rate law '" + name + "'");
+    if (args.size() != (r.law == LAW_MM ? 2u : 3u))
+        throw Error(CWC_E_PARSE, "wrong number of rate-law arguments in '" + t + "'");
+    auto it = atoms.find(args[0]);
+    if (it == atoms.end()) throw Error(CWC_E_INVALID, "unknown atom '" + args[0] + "' in rate law");
+    r.law_atom = it->second;
+    char* end = nullptr;
+    r.law_K = std::strtod(args[1].c_str(), &end);
+    if (args[1].empty() || *end != '\0') throw Error(CWC_E_PARSE, "bad constant in rate law '" + t + "'");
+    if (!std::isfinite(r.law_K) || !(r.law_K > 0))
+        throw Error(CWC_E_INVALID, "rate-law constant must be finite and > 0: '" + t + "'");
+    if (r.law != LAW_MM) {
+        for (char c : args[2])
+            if (!std::isdigit((unsigned char)c)) throw Error(CWC_E_PARSE, "bad Hill exponent in '" + t + "'");
+        if (args[2].empty() || args[2].size() > 2) throw Error(CWC_E_PARSE, "bad Hill exponent in '" + t + "'");
+        r.law_n = std::atoi(args[2].c_str());
+        if (r.law_n < 1 || r.law_n > 8) throw Error(CWC_E_INVALID, "Hill exponent must be in [1, 8]: '" + t + "'");
+    }
+}
+
 Rule parse_rule(const std::string& text, const std::unordered_map<std::string, int>& atoms, double rate) {
     if (!std::isfinite(rate) || rate < 0) throw Error(CWC_E_INVALID, "rate of rule '" + text + "' must be finite and >= 0");
     size_t colon = text.find(':');
@@ -211,6 +252,11 @@ Rule parse_rule(const std::string& text, const std::unordered_map<std::string, i
     r.rate = rate;
     if (!valid_ident(r.label)) throw Error(CWC_E_PARSE, "bad rule label '" + r.label + "'");
     std::string body = text.substr(colon + 1);
+    const size_t at = body.find('@');
+    if (at != std::string::npos) {
+        parse_law(body.substr(at + 1), atoms, r);
+        body = body.substr(0, at);
+    }
     size_t arrow = body.find("->");
     if (arrow == std::string::npos || body.find("->", arrow + 2) != std::string::npos)
         throw Error(CWC_E_PARSE, "rule must contain exactly one '->': '" + text + "'");
@@ -272,6 +318,7 @@ int add_content(std::vector<Region>& regs, const Node& node, const std::string& 
 struct RawReaction {
     int rule;
     double rate;
+    int ctx;  // context region (where a rate law's species is read)
     std::map<std::pair<int, int>, int64_t> react;   // (region, atom) -> order
     std::map<std::pair<int, int>, int64_t> delta;   // (region, atom) -> net change (may be 0)
 };
@@ -358,7 +405,7 @@ FlatModel compile_model(const std::vector<std::string>& alphabet, const std::vec
             std::vector<bool> used(ctx.child_content.size(), false);
             assignments(regs, ctx, rule.lhs.comps, cur, used, found);
             for (const auto& asg : found) {
-                RawReaction rr{(int)ri, rule.rate, {}, {}};
+                RawReaction rr{(int)ri, rule.rate, (int)ci, {}, {}};
                 auto add = [](std::map<std::pair<int, int>, int64_t>& m, int reg, const Counts& c, int64_t sign) {
                     for (size_t a = 0; a < c.size(); ++a)
                         if (c[a]) m[{reg, (int)a}] += sign * c[a];
@@ -392,6 +439,7 @@ FlatModel compile_model(const std::vector<std::string>& alphabet, const std::vec
     for (const auto& rr : raw) {
         for (auto& kv : rr.react) used.insert(kv.first);
         for (auto& kv : rr.delta) used.insert(kv.first);
+        if (parsed[rr.rule].law != LAW_MASS_ACTION) used.insert({rr.ctx, parsed[rr.rule].law_atom});
     }
     if (used.empty()) throw Error(CWC_E_INVALID, "model has no species");
 
@@ -418,6 +466,11 @@ FlatModel compile_model(const std::vector<std::string>& alphabet, const std::vec
         fm.delta.push_back(d);
         fm.rates.push_back(rr.rate);
         fm.rule_of.push_back(rr.rule);
+        const Rule& rule = parsed[rr.rule];
+        fm.law.push_back(rule.law);
+        fm.law_species.push_back(rule.law == LAW_MASS_ACTION ? -1 : sidx[{rr.ctx, rule.law_atom}]);
+        fm.law_K.push_back(rule.law_K);
+        fm.law_n.push_back(rule.law_n);
     }
     fm.x_cap_max = max_exact_cap(fm.reactants, (int64_t)1 << 30);
     return fm;

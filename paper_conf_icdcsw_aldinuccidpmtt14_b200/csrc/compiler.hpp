@@ -21,6 +21,8 @@ struct Error : std::runtime_error {
     Error(int32_t c, const std::string& m) : std::runtime_error(m), code(c) {}
 };
 
+enum Law : int32_t { LAW_MASS_ACTION = 0, LAW_MM = 1, LAW_HILL = 2, LAW_HILLR = 3 };
+
 struct Reactant {
     int32_t species;
     int32_t order;
@@ -35,6 +37,10 @@ struct FlatModel {
     std::vector<std::vector<Reactant>> reactants;  // [M], ascending species
     std::vector<std::vector<int32_t>> delta;     // [M][S]
     std::vector<int32_t> rule_of;                // [M]
+    // functional rate laws (reading R16'): LAW_* per reaction, the species the law reads (-1
+    // for mass action), its constant K and Hill exponent n
+    std::vector<int32_t> law, law_species, law_n;  // [M]
+    std::vector<double> law_K;                     // [M]
     int32_t n_rules = 0;
     int64_t x_cap_max = 0;                       // largest cap with every prod C(cap, r) < 2^53
 

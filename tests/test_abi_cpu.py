@@ -50,6 +50,8 @@ def test_compiler_matches_oracle_flattening(name):
     assert info["rule_of"] == fm.rule_of
     assert info["x_cap"] == fm.x_cap
     assert info["n_rules"] == len(md.rules)
+    assert info["law"] == fm.law and info["law_species"] == fm.law_species
+    assert info["law_K"] == fm.law_K and info["law_n"] == fm.law_n
 
 
 REJECT = [
@@ -67,6 +69,14 @@ REJECT = [
     (["top: A -> B"], [1.0], "(A | .)^top", 1),
     (["top: A -> B"], [1.0], "(A | .", 2),
     (["top: A -> B"], [1.0], "3 A", 2),
+    (["top: A -> B @ mm(A)"], [1.0], "A", 2),                       # rate laws (R16')
+    (["top: A -> B @ hill(A, 3)"], [1.0], "A", 2),
+    (["top: A -> B @ foo(A, 3)"], [1.0], "A", 2),
+    (["top: A -> B @ mm(Q, 3)"], [1.0], "A", 1),
+    (["top: A -> B @ mm(A, -3)"], [1.0], "A", 1),
+    (["top: A -> B @ hill(A, 3, 9)"], [1.0], "A", 1),
+    (["top: A -> B @ hillr(A, 3, 0)"], [1.0], "A", 1),
+    (["top: A -> B @ mm(A, 3"], [1.0], "A", 2),
 ]
 
 

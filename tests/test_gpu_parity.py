@@ -228,3 +228,30 @@ def test_period_analysis_matches_oracle(md, species, lo, hi, t_end, dt, n):
     assert np.array_equal(got["lp_var"], lp_var, equal_nan=True)
     if md is W.CIRCADIAN:   # Vilar oscillator: local period ~ 20-30 h once every instance has one
         assert 20.0 < np.nanmean(lp_mean[-48:]) < 30.0
+
+
+def test_neurospora_rate_laws_parity():
+    """Functional rate laws (MM / Hill) on the paper's Neurospora model."""
+    cfg = W.CONFIGS["neurospora"]
+    _parity(cfg.model, 1200, 48.0, cfg.sample_dt, cfg.seed, first=777, hist_bins=cfg.hist_bins)
+
+
+def test_neurospora_period_analysis_parity():
+    from oracle.period import finalize, period_stats
+    import paper_conf_icdcsw_aldinuccidpmtt14_b200 as cwc
+    pa = W.PERIOD_ANALYSIS["neurospora"]
+    md, n, t_end, dt, seed = W.NEUROSPORA, 2000, 96.0, 0.5, 31
+    m = cwc.Model.from_def(md, hist_bins=64, period_species=pa["species"], period_lo=pa["lo"], period_hi=pa["hi"],
+                           period_window=pa["window"])
+    m.simulate_range(n, 0, n, t_end, dt, seed)
+    m.finalize()
+    got = m.period_stats()
+    fm = flatten_def(md)
+    orun = oracle.simulate(fm, 0, n, t_end, dt, seed, nthreads=16)
+    ps = period_stats(orun.raw, fm.names.index(pa["species"]), pa["lo"], pa["hi"])
+    assert np.array_equal(got["events"], ps.ev) and np.array_equal(got["pc_sum"], ps.pc_sum)
+    assert np.array_equal(got["lp_n"], ps.lp_n) and np.array_equal(got["lp_sum"], ps.lp_sum)
+    lp_mean, ma, lp_var = finalize(ps, dt, pa["window"])
+    assert np.array_equal(got["moving_avg"], ma, equal_nan=True)
+    assert np.array_equal(got["lp_mean"], lp_mean, equal_nan=True)
+    assert 19.0 < ma[-1] < 24.0   # ~21.5 h, the model's published period

@@ -172,3 +172,41 @@ TWO_CELLS = ModelDef(
 
 TINY_MODELS = {m.name: m for m in (PURE_BIRTH, PURE_DEATH, ISOMERIZATION, BINDING, DIMERISATION,
                                    DEAD, RUNAWAY, TRANSPORT, TWO_CELLS)}
+
+# --- functional rate laws ------------------------------------------------------
+# The paper's own workload is the Neurospora circadian model of [20] (PAPER.md P:L323-327,
+# L541-543), whose kinetics are Michaelis-Menten / Hill, not mass action.  Its parameters are
+# not in PAPER.md; these are the published deterministic values of Leloup, Gonze & Goldbeter
+# (J. Biol. Rhythms 1999) [ext], converted to molecule numbers with a system size of 100
+# molecules per nM (the usual stochastic version, Gonze et al. PNAS 2002 [ext]):
+#   dM/dt  = vs KI^n/(KI^n + FN^n) - vm M/(Km + M)
+#   dFC/dt = ks M - vd FC/(Kd + FC) - k1 FC + k2 FN,   dFN/dt = k1 FC - k2 FN
+# vs 1.6, vm 0.505, vd 1.4 nM/h; ks 0.5, k1 0.5, k2 0.6 /h; Km 0.5, Kd 0.13, KI 1 nM; n 4.
+NEUROSPORA = ModelDef(
+    name="neurospora",
+    species=("M", "FC", "FN"),
+    rules=(
+        "top: . -> M @ hillr(FN, 100, 4)",     # frq transcription, repressed by nuclear FRQ
+        "top: M -> . @ mm(M, 50)",             # frq mRNA degradation
+        "top: M -> M FC",                      # translation
+        "top: FC -> . @ mm(FC, 13)",           # cytosolic FRQ degradation
+        "top: FC -> FN",                       # nuclear import
+        "top: FN -> FC",                       # nuclear export
+    ),
+    rates=(160.0, 50.5, 0.5, 140.0, 0.5, 0.6),
+    initial_term=".",
+)
+MODELS[NEUROSPORA.name] = NEUROSPORA
+CONFIGS["neurospora"] = RunConfig(
+    6, NEUROSPORA, 1_000_000, 96.0, 0.5, SEED_BASE + 6, 1024, 1,
+    description="Neurospora circadian model (Leloup-Gonze-Goldbeter, MM/Hill kinetics, 100 molecules/nM), "
+                "1M instances, t_end=96h, dt=0.5h, period analysis on M")
+# period analysis of the paper's experiment: oscillation events of frq mRNA
+PERIOD_ANALYSIS = {"neurospora": dict(species="M", lo=100, hi=350, window=48),
+                   "circadian": dict(species="R", lo=100, hi=1000, window=48)}
+
+# a birth-death chain with Hill-repressed birth and linear death: its stationary law is known in
+# closed form (detailed balance), pinning the functional-rate path of the oracle
+AUTOREPRESSOR = ModelDef("autorepressor", ("P",), ("top: . -> P @ hillr(P, 30, 2)", "top: P -> ."),
+                         (60.0, 1.0), ".")
+TINY_MODELS[AUTOREPRESSOR.name] = AUTOREPRESSOR
