@@ -118,6 +118,7 @@ cwc_status cwc_model_info(cwc_model_t m, cwc_model_info_t* out);
  *   "min_blocks"         register budget: __launch_bounds__ min CTAs per SM; 0 = auto
  *                        (768 / block_threads, i.e. <= 80 registers).
  *   "ilp"                1/2 instances interleaved per thread (ablation knob).      default 1
+ *   "stream"             0/1: on-line streaming — progress counters + cwc_stats_snapshot.
  *   "smem_stats"         0/1: accumulate n/sum/sumsq per CTA in shared memory and flush once
  *                        (used when T*(1+3S)*8 bytes fit without lowering residency). default 1
  *   "seed_jit"           0/1: specialise the kernel on the seed (Philox round keys become
@@ -200,6 +201,17 @@ cwc_status cwc_stats_device(cwc_model_t m, int64_t** dptr, size_t* n_int64);
  * caller into host memory); it must hold stats_len int64 for the last simulated geometry. */
 cwc_status cwc_stats_finalize(cwc_model_t m, const int64_t* host_stats);
 
+/* On-line streaming ("once all simulation tasks overcome a
+ * given simulation time, an array of results is produced and streamed").  With the
+ * option "stream" = 1 the kernel runs in ~16 simulation quanta and counts finished items per
+ * quantum; while it is still running, cwc_stats_snapshot copies the progress counters and then
+ * the statistics through a copy engine on a separate stream (no synchronisation with the
+ * simulation) and derives the cwc_stats views; cuts [0, *cuts_final) of that snapshot are final
+ * (identical to the finished run's), later cuts are partial.  *items_done (optional) = finished
+ * work items.  Moments then accumulate in global memory (no CTA-local staging).
+ * Errors: CWC_E_STATE without a simulation or without "stream". */
+cwc_status cwc_stats_snapshot(cwc_model_t m, int64_t* cuts_final, int64_t* items_done);
+
 typedef struct {
     int32_t T, S, B, n_q;
     const double* times;      /* [T] t_k = fl(k*dt) */
@@ -217,6 +229,7 @@ typedef struct {
     const double* quantile;   /* [T*S*n_q] (+-inf if in the under/overflow bin, NaN if n = 0) */
     int64_t reactions, absorbed, overflowed, finished;
     double kernel_ms;         /* device time of the last simulate kernel (CUDA events) */
+    int64_t cuts_final;       /* cuts [0, cuts_final) are final (T after finalize; see snapshot) */
     const char* const* species_names;
 } cwc_stats_t;
 /* Borrowed views into the handle, valid until the next simulate / finalize / free. */

@@ -45,7 +45,7 @@ class Stats(ctypes.Structure):
                 ("sqlo", P(c_i64)), ("sqhi", P(c_i64)), ("mean", P(c_dbl)), ("var", P(c_dbl)),
                 ("hist", P(c_i64)), ("hist_lo", P(c_i64)), ("hist_width", P(c_i64)), ("q", P(c_dbl)),
                 ("quantile", P(c_dbl)), ("reactions", c_i64), ("absorbed", c_i64), ("overflowed", c_i64),
-                ("finished", c_i64), ("kernel_ms", c_dbl), ("species_names", P(c_cp))]
+                ("finished", c_i64), ("kernel_ms", c_dbl), ("cuts_final", c_i64), ("species_names", P(c_cp))]
 
 
 class PeriodStats(ctypes.Structure):
@@ -72,6 +72,7 @@ SIGNATURES = {
     "cwc_simulate_range": (c_i32, [c_vp, c_i64, c_i64, c_i64, c_dbl, c_dbl, c_u64, c_vp]),
     "cwc_stats_device": (c_i32, [c_vp, P(c_vp), P(c_sz)]),
     "cwc_stats_finalize": (c_i32, [c_vp, c_vp]),
+    "cwc_stats_snapshot": (c_i32, [c_vp, P(c_i64), P(c_i64)]),
     "cwc_stats": (c_i32, [c_vp, P(Stats)]),
     "cwc_samples": (c_i32, [c_vp, c_i64, c_i64, c_vp]),
     "cwc_period_stats": (c_i32, [c_vp, P(PeriodStats)]),

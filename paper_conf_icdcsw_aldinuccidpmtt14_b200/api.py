@@ -48,6 +48,7 @@ class EnsembleResult:
     finished: int
     kernel_ms: float
     species: List[str]
+    cuts_final: int = -1    # cuts [0, cuts_final) are final (T after finalize; a snapshot may be less)
 
     def sumsq_exact(self) -> np.ndarray:
         out = np.empty(self.sqlo.shape, dtype=object)
@@ -223,7 +224,34 @@ class Model:
             quantile=arr(st.quantile, T * S * Q, np.float64, (T, S, Q)) if Q else np.zeros((T, S, 0)),
             reactions=st.reactions, absorbed=st.absorbed, overflowed=st.overflowed, finished=st.finished,
             kernel_ms=st.kernel_ms, species=[st.species_names[s].decode() for s in range(S)],
+            cuts_final=st.cuts_final,
         )
+
+    def snapshot(self):
+        """Statistics of the running simulation ("stream" option): (cuts_final, items_done, result)."""
+        cf, done = ctypes.c_int64(), ctypes.c_int64()
+        check(lib.cwc_stats_snapshot(self._h, ctypes.byref(cf), ctypes.byref(done)))
+        return cf.value, done.value, self.stats()
+
+    def stream(self, n_instances: int, t_end: float, sample_dt: float, seed: int, poll_s: float = 0.02,
+               stream=None):
+        """On-line streaming: launch, then yield (cuts_final, partial result) each
+        time more cuts become final, and finally (T, finalised result)."""
+        import time
+        self.set_option("stream", 1)
+        self.simulate_range(n_instances, 0, n_instances, t_end, sample_dt, seed, stream=stream)
+        last = -1
+        T = int(round(t_end / sample_dt)) + 1
+        while True:
+            cf, _, res = self.snapshot()
+            if cf > last:
+                last = cf
+                if cf < T:
+                    yield cf, res
+            if cf >= T:
+                break
+            time.sleep(poll_s)
+        yield T, self.finalize()
 
     def period_stats(self) -> dict:
         """On-line period analysis of the last simulation (cwc_period_stats) as numpy arrays."""

@@ -189,6 +189,9 @@ cwc_status cwc_set_option_i64(cwc_model_t m, const char* key, int64_t v) {
         } else if (k == "period_window") {
             need(v >= 1 && v <= (int64_t)1 << 30, "period_window >= 1");
             m->period_window = (int)v;
+        } else if (k == "stream") {
+            need(v == 0 || v == 1, "stream is 0 or 1");
+            m->stream = (int)v;
         } else if (k == "smem_stats") {
             need(v == 0 || v == 1, "smem_stats is 0 or 1");
             m->smem_stats = (int)v;
@@ -286,6 +289,13 @@ cwc_status cwc_stats_device(cwc_model_t m, int64_t** dptr, size_t* n) {
     });
 }
 
+cwc_status cwc_stats_snapshot(cwc_model_t m, int64_t* cuts_final, int64_t* items_done) {
+    return guard([&] {
+        need(m != nullptr, "NULL model");
+        cwc::snapshot(m, cuts_final, items_done);
+    });
+}
+
 cwc_status cwc_stats_finalize(cwc_model_t m, const int64_t* host_stats) {
     return guard([&] {
         need(m != nullptr, "NULL model");
@@ -323,6 +333,7 @@ cwc_status cwc_stats(cwc_model_t m, cwc_stats_t* out) {
         out->overflowed = ctr[CWC_CTR_OVERFLOWED];
         out->finished = ctr[CWC_CTR_FINISHED];
         out->kernel_ms = m->kernel_ms;
+        out->cuts_final = m->cuts_final;
         out->species_names = m->name_ptrs.data();
     });
 }

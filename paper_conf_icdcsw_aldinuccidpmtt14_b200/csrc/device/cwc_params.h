@@ -32,6 +32,7 @@ struct cwc_params {
     unsigned long long* st_pd;  // [count] period-detector state (R19)
     unsigned int* st_qdone;     // [count] quanta completed (release/acquire)
     unsigned long long* work;   // work-queue counter
+    unsigned int* qprog;        // [n_quanta] finished items per quantum (streaming progress) or null
     const cwc_logtab_entry* logtab;  // [128]
     long long smem_stats;       // 1: n/sum/sumsq accumulate per CTA in dynamic shared memory
                                 //    (T*(1+3S) u64) and are flushed once at the end

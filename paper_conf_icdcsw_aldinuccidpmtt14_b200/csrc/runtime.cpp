@@ -96,10 +96,10 @@ size_t stats_len(int64_t T, int S, int B, bool period) {
 static size_t align256(size_t v) { return (v + 255) & ~(size_t)255; }
 
 struct ScratchLayout {
-    size_t x, t, step, k, flags, pd, qdone, work, total;
+    size_t x, t, step, k, flags, pd, qdone, work, qprog, total;
 };
 
-static ScratchLayout scratch_layout(int S, int64_t count) {
+static ScratchLayout scratch_layout(int S, int64_t count, int64_t T) {
     ScratchLayout L{};
     size_t off = 0;
     L.x = off; off = align256(off + (size_t)S * count * 4);
@@ -108,9 +108,10 @@ static ScratchLayout scratch_layout(int S, int64_t count) {
     L.step = off; off = align256(off + (size_t)count * 8);
     L.k = off; off = align256(off + (size_t)count * 8);
     L.flags = off; off = align256(off + (size_t)count * 4);
-    L.qdone = off; off += (size_t)count * 4;          // qdone and work are contiguous:
-    off = (off + 7) & ~(size_t)7;                     // one memset clears both
-    L.work = off; off = align256(off + 8);
+    L.qdone = off; off += (size_t)count * 4;          // qdone, work and qprog are contiguous:
+    off = (off + 7) & ~(size_t)7;                     // one memset clears them
+    L.work = off; off += 8;
+    L.qprog = off; off = align256(off + (size_t)T * 4);  // <= T quanta
     L.total = off;
     return L;
 }
@@ -119,7 +120,7 @@ void buffer_sizes(const cwc_model* m, int64_t count, int64_t K, size_t* stats, s
     const int S = m->fm.S();
     if (stats) *stats = stats_len(K + 1, S, m->hist_bins, m->period_species >= 0);
     if (raw) *raw = m->raw_samples ? (size_t)(K + 1) * S * (size_t)count : 0;
-    if (scratch) *scratch = scratch_layout(S, count).total;
+    if (scratch) *scratch = scratch_layout(S, count, K + 1).total;
 }
 
 // ------------------------------------------------------------------------------------ NVRTC
@@ -426,7 +427,8 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     ckd(d.Occupancy(&occ, m->function, m->block_threads, 0), "occupancy");
     if (occ < 1) fail(CWC_E_CUDA, "kernel cannot be resident with block_threads = " + std::to_string(m->block_threads));
     size_t dyn_smem = 0;
-    if (m->smem_stats && mom_bytes <= (size_t)200 * 1024) {
+    // streaming publishes partial statistics while the kernel runs: moments must go to global memory
+    if (m->smem_stats && !m->stream && mom_bytes <= (size_t)200 * 1024) {
         ckd(d.FuncSetAttribute(m->function, CU_FUNC_ATTRIBUTE_MAX_DYNAMIC_SHARED_SIZE_BYTES, (int)mom_bytes),
             "dynamic smem");
         int occ2 = 0;
@@ -444,10 +446,11 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     int64_t qs;
     if (!m->refill) qs = T;  // static assignment: whole trajectories (no cross-lane dependencies)
     else if (m->quantum_samples > 0) qs = std::min<int64_t>(m->quantum_samples, T);
+    else if (m->stream) qs = std::max<int64_t>(1, (T + 15) / 16);  // streaming: progress in ~16 chunks
     else qs = (count >= 4 * lanes) ? (T + 7) / 8 : T;
     const int64_t nq = (T + qs - 1) / qs;
 
-    const ScratchLayout L = scratch_layout(S, count);
+    const ScratchLayout L = scratch_layout(S, count, T);
     char* sc = (char*)m->d_scratch;
     cwc_params P;
     std::memset(&P, 0, sizeof P);
@@ -473,11 +476,12 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     P.st_pd = (unsigned long long*)(sc + L.pd);
     P.st_qdone = (unsigned int*)(sc + L.qdone);
     P.work = (unsigned long long*)(sc + L.work);
+    P.qprog = m->stream ? (unsigned int*)(sc + L.qprog) : nullptr;
     P.logtab = m->d_logtab;
     P.smem_stats = dyn_smem ? 1 : 0;
 
     ck(cudaMemsetAsync(m->d_stats, 0, need_stats * 8, stream), "memset(stats)");
-    ck(cudaMemsetAsync(sc + L.qdone, 0, L.work + 8 - L.qdone, stream), "memset(queue)");
+    ck(cudaMemsetAsync(sc + L.qdone, 0, L.qprog + (size_t)T * 4 - L.qdone, stream), "memset(queue)");
     ck(cudaEventRecord(m->ev0, stream), "cudaEventRecord");
     if (count > 0) {
         void* args[] = {&P};
@@ -522,10 +526,10 @@ static double quantile_from_hist(const int64_t* h, int B, int64_t n, double q, i
     return INFINITY;
 }
 
+static void derive(cwc_model* m);
+
 void finalize(cwc_model* m, const int64_t* host_stats) {
     if (!m->simulated) fail(CWC_E_STATE, "no simulation to finalize");
-    const int64_t T = m->K + 1;
-    const int S = m->fm.S(), B = m->hist_bins;
     const size_t len = m->last_stats_len;
     m->h_stats.resize(len);
     ck(cudaStreamSynchronize(m->last_stream), "simulation");
@@ -533,7 +537,41 @@ void finalize(cwc_model* m, const int64_t* host_stats) {
     if (cudaEventElapsedTime(&ms, m->ev0, m->ev1) == cudaSuccess) m->kernel_ms = ms;
     if (host_stats) std::memcpy(m->h_stats.data(), host_stats, len * 8);
     else ck(cudaMemcpy(m->h_stats.data(), m->d_stats, len * 8, cudaMemcpyDeviceToHost), "copy stats");
+    m->cuts_final = m->K + 1;
+    derive(m);
+}
 
+// On-line streaming: while the kernel
+// runs, read the per-quantum progress counters and then the statistics through a copy engine on
+// a separate stream.  Cuts below (q+1)*qs are final once every item of quanta 0..q has finished
+// (an instance that ended early emitted or filled all its later cuts).  The counters are read
+// before the statistics, so the snapshot contains every update of the cuts it reports final.
+void snapshot(cwc_model* m, int64_t* cuts_final, int64_t* items_done) {
+    if (!m->simulated) fail(CWC_E_STATE, "no simulation");
+    if (!m->stream) fail(CWC_E_STATE, "snapshots need the \"stream\" option set before simulating");
+    if (!m->poll_stream) ck(cudaStreamCreateWithFlags(&m->poll_stream, cudaStreamNonBlocking), "cudaStreamCreate");
+    const int64_t T = m->K + 1, nq = (T + m->qs - 1) / m->qs;
+    const ScratchLayout L = scratch_layout(m->fm.S(), m->count, T);
+    std::vector<uint32_t> prog((size_t)nq);
+    ck(cudaMemcpyAsync(prog.data(), (const char*)m->d_scratch + L.qprog, nq * 4, cudaMemcpyDeviceToHost,
+                       m->poll_stream), "copy progress");
+    ck(cudaStreamSynchronize(m->poll_stream), "copy progress");
+    int64_t q = 0, done = 0;
+    while (q < nq && prog[q] >= (uint64_t)m->count) ++q;
+    for (uint32_t v : prog) done += v;
+    m->h_stats.resize(m->last_stats_len);
+    ck(cudaMemcpyAsync(m->h_stats.data(), m->d_stats, m->last_stats_len * 8, cudaMemcpyDeviceToHost, m->poll_stream),
+       "copy stats");
+    ck(cudaStreamSynchronize(m->poll_stream), "copy stats");
+    m->cuts_final = std::min<int64_t>(q * m->qs, T);
+    derive(m);
+    if (cuts_final) *cuts_final = m->cuts_final;
+    if (items_done) *items_done = done;
+}
+
+static void derive(cwc_model* m) {
+    const int64_t T = m->K + 1;
+    const int S = m->fm.S(), B = m->hist_bins;
     const int64_t* p = m->h_stats.data();
     const int64_t TS = T * S;
     m->h_n.assign(p, p + T);
@@ -613,7 +651,7 @@ void copy_records(cwc_model* m, int64_t first, int64_t count, uint8_t* flags, in
     if (first < 0 || count < 0 || first + count > m->count) fail(CWC_E_INVALID, "range outside the last simulation");
     ck(cudaStreamSynchronize(m->last_stream), "simulation");
     if (count == 0) return;
-    const ScratchLayout L = scratch_layout(m->fm.S(), m->count);
+    const ScratchLayout L = scratch_layout(m->fm.S(), m->count, m->K + 1);
     const char* sc = (const char*)m->d_scratch;
     if (flags) {
         std::vector<uint32_t> f(count);
@@ -635,6 +673,7 @@ cwc_model::~cwc_model() {
     cwc::free_owned(this);
     if (d_logtab) cudaFree(d_logtab);
     if (own_stream) cudaStreamDestroy(own_stream);
+    if (poll_stream) cudaStreamDestroy(poll_stream);
     if (ev0) cudaEventDestroy(ev0);
     if (ev1) cudaEventDestroy(ev1);
 }

@@ -30,6 +30,9 @@ struct cwc_model {
     int period_species = -1;
     int64_t period_lo = 0, period_hi = 1;
     int period_window = 1;
+    int stream = 0;                       // on-line streaming: progress counters + snapshots
+    cudaStream_t poll_stream = nullptr;   // copy-engine stream for snapshots
+    int64_t cuts_final = 0;               // cuts final in the host views (T after finalize)
     int blocks_per_sm = 0;
     int refill = 1;
     int device = -1;
@@ -90,6 +93,7 @@ void compile(cwc_model* m, const uint64_t* seed = nullptr);  // NVRTC (no GPU ne
 void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count, double t_end, double dt,
                     uint64_t seed, cudaStream_t stream, bool own_stream = false);
 void finalize(cwc_model* m, const int64_t* host_stats);
+void snapshot(cwc_model* m, int64_t* cuts_final, int64_t* items_done);
 void bind_buffers(cwc_model* m, int64_t* stats, size_t stats_n, int32_t* raw, size_t raw_n, void* scratch,
                   size_t scratch_bytes);
 void copy_samples(cwc_model* m, int64_t first, int64_t count, int32_t* out);

@@ -255,3 +255,30 @@ def test_neurospora_period_analysis_parity():
     assert np.array_equal(got["moving_avg"], ma, equal_nan=True)
     assert np.array_equal(got["lp_mean"], lp_mean, equal_nan=True)
     assert 19.0 < ma[-1] < 24.0   # ~21.5 h, the model's published period
+
+
+# ------------------------------------------------------------------ on-line streaming (§8(f)-2)
+def test_streaming_snapshots_are_final_prefixes():
+    """Snapshots taken while the kernel runs: the cuts they report final equal the finished run."""
+    import paper_conf_icdcsw_aldinuccidpmtt14_b200 as cwc
+    cfg = W.CONFIGS["schlogl"]
+    n, t_end = 200_000, 20.0
+    m = cwc.Model.from_def(cfg.model, hist_bins=cfg.hist_bins, raw_samples=False)
+    snaps = [(cf, res) for cf, res in m.stream(n, t_end, cfg.sample_dt, cfg.seed, poll_s=0.005)]
+    final = snaps[-1][1]
+    T = final.n.size
+    assert snaps[-1][0] == T and final.finished == n
+    partial = [(cf, r) for cf, r in snaps[:-1] if cf > 0]
+    assert len(partial) >= 2, [cf for cf, _ in snaps]          # progress was observed mid-run
+    prev = 0
+    for cf, r in partial:
+        assert prev <= cf < T
+        prev = cf
+        for name in ("n", "sum", "sqlo", "sqhi", "hist"):
+            assert np.array_equal(getattr(r, name)[:cf], getattr(final, name)[:cf]), (cf, name)
+        assert np.array_equal(r.mean[:cf], final.mean[:cf], equal_nan=True)
+    # and the streamed run equals a normal run
+    ref = cwc.Model.from_def(cfg.model, hist_bins=cfg.hist_bins, raw_samples=False).simulate(
+        n, t_end, cfg.sample_dt, cfg.seed)
+    for name in ("n", "sum", "sqlo", "sqhi", "hist"):
+        assert np.array_equal(getattr(ref, name), getattr(final, name))
