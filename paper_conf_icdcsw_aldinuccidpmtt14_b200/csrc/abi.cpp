@@ -189,6 +189,9 @@ cwc_status cwc_set_option_i64(cwc_model_t m, const char* key, int64_t v) {
         } else if (k == "period_window") {
             need(v >= 1 && v <= (int64_t)1 << 30, "period_window >= 1");
             m->period_window = (int)v;
+        } else if (k == "delta_table") {
+            need(v >= -1 && v <= 1, "delta_table is -1 (auto), 0 or 1");
+            m->delta_table = (int)v;
         } else if (k == "stream") {
             need(v == 0 || v == 1, "stream is 0 or 1");
             m->stream = (int)v;

@@ -117,18 +117,63 @@ std::string generate_model_section(const FlatModel& fm, const KernelConfig& cfg)
     o << "    if (j >= CWC_M) j = cwc_last_positive(x);\n";
     o << "    return j;\n}\n\n";
 
-    // rewrite + overflow check on the species some rule increases
-    o << "__device__ __forceinline__ bool cwc_apply(int j, int (&x)[CWC_S]) {\n";
+    // rewrite + overflow check on the species some rule increases.  Few (rule, species) pairs:
+    // a predicated select chain; many (large networks): the selected rule's row of packed int8
+    // deltas from a shared-memory table (one vector load + a sign-extending byte extract per species)
     std::vector<bool> inc(S, false);
-    for (int s = 0; s < S; ++s) {
-        std::string chain = "0";
-        for (int j = M - 1; j >= 0; --j) {
-            int d = fm.delta[j][s];
-            if (!d) continue;
-            if (d > 0) inc[s] = true;
-            chain = "(j == " + std::to_string(j) + " ? " + std::to_string(d) + " : " + chain + ")";
+    int pairs = 0, maxabs = 0;
+    for (int j = 0; j < M; ++j)
+        for (int s = 0; s < S; ++s)
+            if (fm.delta[j][s]) {
+                ++pairs;
+                maxabs = std::max(maxabs, std::abs(fm.delta[j][s]));
+                if (fm.delta[j][s] > 0) inc[s] = true;
+            }
+    const bool table = (cfg.delta_table == 1 || (cfg.delta_table < 0 && pairs > 2 * S)) && maxabs <= 127 && M > 0;
+    const int words = (S + 3) / 4, wpad = words <= 1 ? 1 : (words <= 2 ? 2 : (words + 3) / 4 * 4);
+    if (table) {
+        o << "#define CWC_DELTA_TABLE 1\n#define CWC_DELTA_WORDS " << wpad << "\n";
+        o << "__constant__ unsigned int cwc_delta_const[" << M * wpad << "] = {";
+        for (int j = 0; j < M; ++j)
+            for (int w = 0; w < wpad; ++w) {
+                uint32_t word = 0;
+                for (int b = 0; b < 4; ++b) {
+                    const int s = w * 4 + b;
+                    if (s < S) word |= (uint32_t)(uint8_t)(int8_t)fm.delta[j][s] << (8 * b);
+                }
+                o << (j || w ? ", " : "") << word << "u";
+            }
+        o << "};\n__shared__ __align__(16) unsigned int cwc_delta_smem[" << M * wpad << "];\n";
+        o << "__device__ __forceinline__ void cwc_delta_init() {\n    for (int i = threadIdx.x; i < "
+          << M * wpad << "; i += blockDim.x) cwc_delta_smem[i] = cwc_delta_const[i];\n}\n";
+        o << "__device__ __forceinline__ bool cwc_apply(int j, int (&x)[CWC_S]) {\n";
+        o << "    const unsigned int* row = cwc_delta_smem + j * CWC_DELTA_WORDS;\n";
+        o << "    unsigned int w[CWC_DELTA_WORDS];\n";
+        if (wpad == 1) o << "    w[0] = row[0];\n";
+        else if (wpad == 2) o << "    { const uint2 v = *reinterpret_cast<const uint2*>(row); w[0] = v.x; w[1] = v.y; }\n";
+        else
+            for (int q = 0; q < wpad / 4; ++q)
+                o << "    { const uint4 v = *reinterpret_cast<const uint4*>(row + " << 4 * q << "); w[" << 4 * q
+                  << "] = v.x; w[" << 4 * q + 1 << "] = v.y; w[" << 4 * q + 2 << "] = v.z; w[" << 4 * q + 3
+                  << "] = v.w; }\n";
+        for (int s = 0; s < S; ++s) {
+            bool any = false;
+            for (int j = 0; j < M; ++j) any |= fm.delta[j][s] != 0;
+            if (any)
+                o << "    x[" << s << "] += ((int)(w[" << s / 4 << "] << " << 24 - 8 * (s % 4) << ")) >> 24;\n";
         }
-        if (chain != "0") o << "    x[" << s << "] += " << chain << ";\n";
+    } else {
+        o << "__device__ __forceinline__ void cwc_delta_init() {}\n";
+        o << "__device__ __forceinline__ bool cwc_apply(int j, int (&x)[CWC_S]) {\n";
+        for (int s = 0; s < S; ++s) {
+            std::string chain = "0";
+            for (int j = M - 1; j >= 0; --j) {
+                int d = fm.delta[j][s];
+                if (!d) continue;
+                chain = "(j == " + std::to_string(j) + " ? " + std::to_string(d) + " : " + chain + ")";
+            }
+            if (chain != "0") o << "    x[" << s << "] += " << chain << ";\n";
+        }
     }
     o << "    bool over = false;\n";
     for (int s = 0; s < S; ++s)

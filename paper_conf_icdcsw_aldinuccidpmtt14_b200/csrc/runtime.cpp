@@ -222,6 +222,7 @@ void compile(cwc_model* m, const uint64_t* seed) {
     // App. B models (fewer, fatter threads lose more to latency than they gain from registers)
     cfg.min_blocks = m->min_blocks > 0 ? m->min_blocks : std::max(1, 768 / m->block_threads);
     cfg.ilp = m->ilp;
+    cfg.delta_table = m->delta_table;
     cfg.period_species = m->period_species;
     cfg.period_lo = m->period_lo;
     cfg.period_hi = m->period_hi;

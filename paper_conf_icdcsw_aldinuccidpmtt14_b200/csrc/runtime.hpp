@@ -24,6 +24,7 @@ struct cwc_model {
     int block_threads = 256;
     int min_blocks = 0;
     int ilp = 1;
+    int delta_table = -1;
     int smem_stats = 1;
     // on-line period analysis (reading R19): observable species (-1 = off), Schmitt thresholds,
     // moving-average window in cuts

@@ -1,0 +1,44 @@
+"""Small runs of every model for compute-sanitizer (memcheck / racecheck / synccheck):
+
+    compute-sanitizer --tool memcheck python tools/sanitize_run.py
+
+Exercises quanta + refill, raw cuts, overflow fill, absorption, period analysis, rate laws,
+streaming snapshots and the shared-memory moment staging.
+"""
+import os
+import sys
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+sys.path.insert(0, ROOT)
+
+import workloads as W  # noqa: E402
+import paper_conf_icdcsw_aldinuccidpmtt14_b200 as cwc  # noqa: E402
+
+
+def main():
+    # sizes keep every run under ~1e6 reactions: the sanitizers slow kernels down 100-1000x
+    runs = [
+        (W.IMM_DEATH, 300, 10.0, 1.0, {}),
+        (W.LOTKA_VOLTERRA, 300, 0.3, 0.05, {"quantum_samples": 2}),
+        (W.SCHLOGL, 500, 0.5, 0.05, {"quantum_samples": 2, "block_threads": 128}),
+        (W.CIRCADIAN, 200, 4.0, 0.5, {"period_species": "R", "period_lo": 100, "period_hi": 1000}),
+        (W.COMPARTMENTS, 200, 2.0, 0.5, {"smem_stats": 0}),
+        (W.NEUROSPORA, 200, 6.0, 0.5, {"period_species": "M", "period_lo": 100, "period_hi": 350}),
+        (W.RUNAWAY, 100, 10.0, 0.5, {}),
+        (W.DEAD, 100, 3.0, 0.5, {}),
+    ]
+    for md, n, t_end, dt, opts in runs:
+        m = cwc.Model.from_def(md, hist_bins=64, **opts)
+        res = m.simulate(n, t_end, dt, 123)
+        assert res.finished == n, md.name
+        if "period_species" in opts:
+            m.period_stats()
+        print(f"{md.name}: {res.reactions} reactions ok", flush=True)
+    m = cwc.Model.from_def(W.SCHLOGL, hist_bins=64, raw_samples=False)
+    for cf, res in m.stream(2000, 0.5, 0.05, 7, poll_s=0.001):
+        pass
+    print("stream ok", flush=True)
+
+
+if __name__ == "__main__":
+    main()
