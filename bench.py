@@ -339,7 +339,7 @@ def run_b200(args):
                     "d2h_bytes_per_step": n_stats * 8, "ms_per_step": float(te[0]),
                     "path": "dist.simulate_sharded (public API): launch + all-reduce + D2H stats + finalize"},
             "clocks": clk,
-            "kernel": {**model.kernel_attributes(), "block": 256, "load_s": load_s},
+            "kernel": {**model.kernel_attributes(), "load_s": load_s},
             "stats_check": {"finished": res.finished, "absorbed": res.absorbed, "overflowed": res.overflowed},
         }
         print(json.dumps(line), flush=True)

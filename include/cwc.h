@@ -113,7 +113,7 @@ cwc_status cwc_model_info(cwc_model_t m, cwc_model_info_t* out);
  *   "hist_lo"            left edge of bin 1 for every species; "hist_lo.<species name>" for one.
  *   "quantum_samples"    sample points per simulation quantum (Q/tau); 0 = auto.
  *                        Scheduling only: results are bit-identical for every value (R12).
- *   "block_threads"      CUDA block size (multiple of 32, <= 1024).              default 256
+ *   "block_threads"      CUDA block size (multiple of 32, <= 1024).              default 768
  *   "blocks_per_sm"      persistent CTAs per SM; 0 = occupancy maximum.          default 0
  *   "min_blocks"         register budget: __launch_bounds__ min CTAs per SM; 0 = auto
  *                        (768 / block_threads, i.e. <= 80 registers).
