@@ -190,7 +190,7 @@ cwc_status cwc_set_option_i64(cwc_model_t m, const char* key, int64_t v) {
             need(v >= 1 && v <= (int64_t)1 << 30, "period_window >= 1");
             m->period_window = (int)v;
         } else if (k == "delta_table") {
-            need(v >= -1 && v <= 1, "delta_table is -1 (auto), 0 or 1");
+            need(v >= -1 && v <= 2, "delta_table is -1 (auto), 0 (select chain), 1 (table) or 2 (telescoped)");
             m->delta_table = (int)v;
         } else if (k == "stream") {
             need(v == 0 || v == 1, "stream is 0 or 1");

@@ -130,6 +130,33 @@ std::string generate_model_section(const FlatModel& fm, const KernelConfig& cfg)
                 if (fm.delta[j][s] > 0) inc[s] = true;
             }
     const bool table = (cfg.delta_table == 1 || (cfg.delta_table < 0 && pairs > 2 * S)) && maxabs <= 127 && M > 0;
+    // fast-path rewrite straight from the selection predicates p_i = (cum_i <= target), which are
+    // monotone (cum is non-decreasing), so p_i = [i < j*] and the telescoping sum
+    // nu_0 + sum_{i<M-1} (nu_{i+1} - nu_i) p_i = nu_{j*} needs no rule index at all
+    const bool telescope = !table && M > 1 && (cfg.delta_table == 2 || cfg.delta_table < 0);
+    if (telescope) {
+        o << "#define CWC_TELESCOPE 1\n";
+        o << "__device__ __forceinline__ bool cwc_apply_p(const bool (&p)[CWC_M], int (&x)[CWC_S]) {\n";
+        for (int s = 0; s < S; ++s) {
+            const int base = fm.delta[0][s];
+            std::vector<std::pair<int, int>> terms;  // (i, nu_{i+1,s} - nu_{i,s})
+            for (int i = 0; i + 1 < M; ++i)
+                if (fm.delta[i + 1][s] != fm.delta[i][s]) terms.push_back({i, fm.delta[i + 1][s] - fm.delta[i][s]});
+            if (terms.empty() && base == 0) continue;
+            std::string e;
+            for (size_t t = 0; t < terms.size(); ++t) {
+                const int d = terms[t].second + (t == 0 ? base : 0), z = (t == 0 ? base : 0);
+                e += (t ? " + " : "") + std::string("(p[") + std::to_string(terms[t].first) + "] ? " + std::to_string(d) +
+                     " : " + std::to_string(z) + ")";
+            }
+            if (terms.empty()) e = std::to_string(base);
+            o << "    x[" << s << "] += " << e << ";\n";
+        }
+        o << "    bool over = false;\n";
+        for (int s = 0; s < S; ++s)
+            if (inc[s]) o << "    over |= x[" << s << "] > CWC_X_CAP;\n";
+        o << "    return over;\n}\n\n";
+    }
     const int words = (S + 3) / 4, wpad = words <= 1 ? 1 : (words <= 2 ? 2 : (words + 3) / 4 * 4);
     if (table) {
         o << "#define CWC_DELTA_TABLE 1\n#define CWC_DELTA_WORDS " << wpad << "\n";

@@ -12,7 +12,7 @@ struct KernelConfig {
     int block_threads = 256;
     int min_blocks = 0;  // __launch_bounds__ min blocks per SM (0 = let ptxas choose)
     int ilp = 1;         // instances per thread
-    int delta_table = -1;  // rewrite via a shared-memory delta table: 1 yes, 0 no, -1 auto
+    int delta_table = -1;  // rewrite: 1 shared-memory delta table, 0 select chain, 2 telescoped predicates, -1 auto
     int hist_bins = 256;
     bool seed_keys = false;  // bake the Philox round keys of `seed` into the kernel (immediates)
     uint64_t seed = 0;
