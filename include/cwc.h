@@ -37,15 +37,17 @@ typedef int32_t cwc_status;
 #define CWC_OK 0
 #define CWC_E_INVALID 1     /* bad argument / value (null, negative, NaN, unknown atom, ...) */
 #define CWC_E_PARSE 2       /* syntax error in a term or rule */
-#define CWC_E_UNSUPPORTED 3 /* valid CWC outside the hot path: compartment creation/destruction,
-                               reaction order > 3, closed membrane patterns, moved variables */
+#define CWC_E_UNSUPPORTED 3 /* valid CWC outside the hot path: reaction order > 3, closed
+                               membrane patterns, moved variables, nested dynamic compartments,
+                               more than one compartment created by a rule (reading R20) */
 #define CWC_E_CUDA 4        /* CUDA / NVRTC / driver failure, or no device */
 #define CWC_E_OOM 5         /* device allocation failed */
 #define CWC_E_STATE 6       /* call out of order (e.g. stats before any simulation) */
 
 /* Per-instance flags (reading R8/R9). 0 = reached t_end. */
 #define CWC_FLAG_ABSORBED 1   /* a0 == 0: state held to t_end */
-#define CWC_FLAG_OVERFLOWED 2 /* a count exceeded x_cap: frozen, later samples missing (-1) */
+#define CWC_FLAG_OVERFLOWED 2 /* a count exceeded x_cap, or a compartment pool was full when a
+                                 rule created a compartment (R20): frozen, later samples -1 */
 
 typedef struct cwc_model* cwc_model_t;
 
@@ -60,6 +62,15 @@ typedef struct cwc_model* cwc_model_t;
  *   initial_term e.g. "500*L (100*R | (. | 2*G)^nuc)^cell".
  * The static compartment structure is flattened at load (DESIGN.md §3 "flattening"): one flat
  * species per (region, atom), one flat reaction per (rule, context, compartment assignment).
+ * Dynamic compartments (reading R20): a rule may create one compartment, written as
+ * a ground rhs compartment "(wrap | content)^label" without variables, and may destroy pattern
+ * compartments that do not reappear on its rhs; "$x" / "$X" of a destroyed compartment written
+ * at rule level on the rhs release its remaining wrap / content into the rule's context, else
+ * they vanish.  Compartments of a label some rule creates or destroys ("dynamic" labels) are
+ * leaves (atoms only) and live in bounded pools: capacity.<label> slots (default 8) per region
+ * that holds them, each slot with an occupancy flag species "#alive@<path>", each pool with a
+ * free-slot counter "#free:<label>[@<path>]"; a creation takes the lowest free slot, and a
+ * creation at a full pool sets "#full" and freezes the instance as CWC_FLAG_OVERFLOWED.
  * *out receives a library-owned handle (free with cwc_model_free).
  * Errors: CWC_E_INVALID, CWC_E_PARSE, CWC_E_UNSUPPORTED.
  * ---------------------------------------------------------------------------------------- */
@@ -74,9 +85,22 @@ void cwc_model_free(cwc_model_t m);
 const char* cwc_last_error(void);
 
 /* Flat view of a loaded model.  All pointers are borrowed views owned by the handle, valid
- * until cwc_model_free (or a cwc_set_option that changes x_cap / histogram layout).
- *   reactant_species/order: [n_reactions][4], entries beyond n_reactants[j] are 0.
- *   delta: [n_reactions][n_species] dense net change nu_j (row-major). */
+ * until cwc_model_free (or a cwc_set_option that changes x_cap / histogram layout / capacity).
+ *   reactant_species/order: [n_reactions][CWC_MAX_REACTANTS], entries beyond n_reactants[j]
+ *                           are 0.
+ *   delta: [n_reactions][n_species] dense net change nu_j (row-major).
+ * Reading R20 (dynamic compartments; see cwc_model_load), per flat reaction j:
+ *   gate_species[j]/gate_kind[j]  -1/0, or a species g with kind 1 (enabled while x_g >= 1: a
+ *                                 creation) or 2 (enabled while x_g == 0: its pool is full);
+ *                                 the propensity is multiplied by that 0/1 condition.
+ *   place_off[j]..place_off[j+1]  candidate slots of a creation, in order: slot p has the
+ *                                 occupancy flag place_alive[p] and the additions
+ *                                 add_species/add_count[add_off[p]..add_off[p+1]); after
+ *                                 x += nu_j the first slot with flag 0 receives its additions.
+ *   xfer_off[j]..xfer_off[j+1]    moves of a destruction, after x += nu_j: x[xfer_dst] +=
+ *                                 x[xfer_src] (xfer_dst >= 0), then x[xfer_src] = 0.
+ *   sentinel                      species "#full" or -1; flag[s] = 1 for occupancy flags. */
+#define CWC_MAX_REACTANTS 8
 typedef struct {
     int32_t n_species;
     int32_t n_reactions;
@@ -101,11 +125,26 @@ typedef struct {
     const int32_t* law_species;
     const double* law_K;
     const int32_t* law_n;
+    const int32_t* gate_species;      /* [n_reactions] (R20) */
+    const int32_t* gate_kind;
+    const int32_t* place_off;         /* [n_reactions + 1] */
+    const int32_t* place_alive;       /* [place_off[n_reactions]] */
+    const int32_t* add_off;           /* [place_off[n_reactions] + 1] */
+    const int32_t* add_species;
+    const int32_t* add_count;
+    const int32_t* xfer_off;          /* [n_reactions + 1] */
+    const int32_t* xfer_src;
+    const int32_t* xfer_dst;
+    int32_t sentinel;
+    const uint8_t* flag;              /* [n_species] */
 } cwc_model_info_t;
 cwc_status cwc_model_info(cwc_model_t m, cwc_model_info_t* out);
 
 /* ------------------------------------------------------------------------------------------
  * Options (cwc_set_option_i64 unless noted).  Keys:
+ *   "capacity.<label>"   slots per pool of a dynamic compartment label, [1, 4096] (R20).
+ *                        Re-flattens the model: set it first (species-indexed options such as
+ *                        hist_width.<name>, period_species and x_cap are reset).   default 8
  *   "x_cap"              1 <= v <= x_cap_max (R9).                       default x_cap_max or model's
  *   "raw_samples"        0/1: keep the raw [T][S][count] int32 sample buffer.   default 1
  *   "hist_bins"          B >= 1 in-range bins per (time, species).               default 256

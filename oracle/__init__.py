@@ -57,7 +57,20 @@ class _Model(ctypes.Structure):
         ("law_s", ctypes.POINTER(ctypes.c_int32)),
         ("law_K", ctypes.POINTER(ctypes.c_double)),
         ("law_n", ctypes.POINTER(ctypes.c_int32)),
+        ("gate_s", ctypes.POINTER(ctypes.c_int32)),
+        ("gate_k", ctypes.POINTER(ctypes.c_int32)),
+        ("place_off", ctypes.POINTER(ctypes.c_int32)),
+        ("place_alive", ctypes.POINTER(ctypes.c_int32)),
+        ("add_off", ctypes.POINTER(ctypes.c_int32)),
+        ("add_s", ctypes.POINTER(ctypes.c_int32)),
+        ("add_n", ctypes.POINTER(ctypes.c_int32)),
+        ("xfer_off", ctypes.POINTER(ctypes.c_int32)),
+        ("xfer_src", ctypes.POINTER(ctypes.c_int32)),
+        ("xfer_dst", ctypes.POINTER(ctypes.c_int32)),
+        ("sentinel", ctypes.c_int32),
     ]
+
+RMAX = 8  # reactant entries per flat reaction (ORACLE_RMAX in ssa.c)
 
 
 _lib = None
@@ -116,24 +129,41 @@ class CModel:
         self.x0 = np.array(fm.x0, dtype=np.int32)
         self.k = np.array(fm.rates, dtype=np.float64) if M else np.zeros(1)
         self.n_react = np.array([len(r) for r in fm.reactants] or [0], dtype=np.int32)
-        self.react_s = np.zeros(max(M, 1) * 4, dtype=np.int32)
-        self.react_r = np.zeros(max(M, 1) * 4, dtype=np.int32)
+        self.react_s = np.zeros(max(M, 1) * RMAX, dtype=np.int32)
+        self.react_r = np.zeros(max(M, 1) * RMAX, dtype=np.int32)
         for j, rl in enumerate(fm.reactants):
+            if len(rl) > RMAX:
+                raise CWCError("unsupported", f"flat reaction {j} has more than {RMAX} reactant species")
             for e, (s, r) in enumerate(rl):
-                self.react_s[j * 4 + e] = s
-                self.react_r[j * 4 + e] = r
+                self.react_s[j * RMAX + e] = s
+                self.react_r[j * RMAX + e] = r
         self.delta = np.array(fm.delta, dtype=np.int32).reshape(-1) if M else np.zeros(1, np.int32)
         nz = max(M, 1)
         self.law = np.array(fm.law or [0] * nz, dtype=np.int32)
         self.law_s = np.array(fm.law_species or [-1] * nz, dtype=np.int32)
         self.law_K = np.array(fm.law_K or [0.0] * nz, dtype=np.float64)
         self.law_n = np.array(fm.law_n or [1] * nz, dtype=np.int32)
+        # reading R20: gates, creations (place), destructions (transfer), the "#full" sentinel
+        self.gate_s = np.array(fm.gate_species or [-1] * nz, dtype=np.int32)
+        self.gate_k = np.array(fm.gate_kind or [0] * nz, dtype=np.int32)
+        place = fm.place or [[] for _ in range(M)]
+        xfer = fm.transfer or [[] for _ in range(M)]
+        self.place_off = np.cumsum([0] + [len(p) for p in place]).astype(np.int32)
+        self.place_alive = np.array([al for p in place for al, _ in p] or [0], dtype=np.int32)
+        self.add_off = np.cumsum([0] + [len(ad) for p in place for _, ad in p]).astype(np.int32)
+        self.add_s = np.array([sp for p in place for _, ad in p for sp, _ in ad] or [0], dtype=np.int32)
+        self.add_n = np.array([n for p in place for _, ad in p for _, n in ad] or [0], dtype=np.int32)
+        self.xfer_off = np.cumsum([0] + [len(x) for x in xfer]).astype(np.int32)
+        self.xfer_src = np.array([a for x in xfer for a, _ in x] or [0], dtype=np.int32)
+        self.xfer_dst = np.array([b for x in xfer for _, b in x] or [0], dtype=np.int32)
         P = lambda a, t: a.ctypes.data_as(ctypes.POINTER(t))  # noqa: E731
-        self.c = _Model(S, M, P(self.x0, ctypes.c_int32), P(self.k, ctypes.c_double),
-                        P(self.n_react, ctypes.c_int32), P(self.react_s, ctypes.c_int32),
-                        P(self.react_r, ctypes.c_int32), P(self.delta, ctypes.c_int32), fm.x_cap,
-                        P(self.law, ctypes.c_int32), P(self.law_s, ctypes.c_int32),
-                        P(self.law_K, ctypes.c_double), P(self.law_n, ctypes.c_int32))
+        I = lambda a: P(a, ctypes.c_int32)  # noqa: E731
+        self.c = _Model(S, M, I(self.x0), P(self.k, ctypes.c_double),
+                        I(self.n_react), I(self.react_s), I(self.react_r), I(self.delta), fm.x_cap,
+                        I(self.law), I(self.law_s), P(self.law_K, ctypes.c_double), I(self.law_n),
+                        I(self.gate_s), I(self.gate_k), I(self.place_off), I(self.place_alive),
+                        I(self.add_off), I(self.add_s), I(self.add_n), I(self.xfer_off), I(self.xfer_src),
+                        I(self.xfer_dst), int(fm.sentinel))
 
     def propensities(self, x):
         x = np.ascontiguousarray(x, dtype=np.int32)

@@ -140,15 +140,31 @@ typedef struct {
     const int32_t* x0;       /* [S] */
     const double* k;         /* [M] rate constants */
     const int32_t* n_react;  /* [M] number of (species, order) reactant entries */
-    const int32_t* react_s;  /* [M*4] reactant species */
-    const int32_t* react_r;  /* [M*4] reactant orders (stoichiometric coefficient) */
+    const int32_t* react_s;  /* [M*ORACLE_RMAX] reactant species */
+    const int32_t* react_r;  /* [M*ORACLE_RMAX] reactant orders (stoichiometric coefficient) */
     const int32_t* delta;    /* [M*S] dense net change nu_j */
     int64_t x_cap;           /* reading R9 */
     const int32_t* law;      /* [M] 0 mass action, 1 mm, 2 hill, 3 hillr (reading R16') */
     const int32_t* law_s;    /* [M] species the law reads */
     const double* law_K;     /* [M] */
     const int32_t* law_n;    /* [M] Hill exponent */
+    /* reading R20 (dynamic compartments in bounded pools); all may be NULL for static models */
+    const int32_t* gate_s;   /* [M] species gating the reaction, -1 none */
+    const int32_t* gate_k;   /* [M] 1: enabled while x >= 1, 2: enabled while x == 0 */
+    const int32_t* place_off;    /* [M+1] candidate slots of a creation: place_alive[off[j]..off[j+1]) */
+    const int32_t* place_alive;  /* [P] occupancy flag species of each candidate slot */
+    const int32_t* add_off;      /* [P+1] additions of a slot: add_s/add_n[add_off[p]..add_off[p+1]) */
+    const int32_t* add_s;
+    const int32_t* add_n;
+    const int32_t* xfer_off;     /* [M+1] moves of a destruction: xfer_src/dst[xfer_off[j]..) */
+    const int32_t* xfer_src;
+    const int32_t* xfer_dst;     /* -1: removed */
+    int32_t sentinel;            /* species "#full" (> 0 = a pool overflowed), -1 none */
 } oracle_model;
+
+#define ORACLE_RMAX 8   /* reactant entries per flat reaction */
+#define ORACLE_SMAX 512 /* species */
+#define ORACLE_MMAX 4096 /* flat reactions */
 
 enum { ORACLE_FLAG_ABSORBED = 1, ORACLE_FLAG_OVERFLOWED = 2 };
 
@@ -175,6 +191,12 @@ static double ipow(double y, int n) {
 
 static double propensity(const oracle_model* m, int32_t j, const int32_t* x, uint64_t h) {
     const int law = m->law ? m->law[j] : 0;
+    /* reading R20: a creation is enabled while its pool has a free slot (gate x >= 1), the
+     * pool-full reaction while it has none (gate x == 0) */
+    if (m->gate_s && m->gate_s[j] >= 0) {
+        const int32_t g = x[m->gate_s[j]];
+        if (m->gate_k[j] == 1 ? g < 1 : g != 0) h = 0;
+    }
     if (law == 0) return m->k[j] * (double)h;
     if (h == 0) return 0.0;
     const double X = (double)x[m->law_s[j]], K = m->law_K[j];
@@ -214,8 +236,8 @@ static void simulate_instance(const job_t* jb, int64_t li) {
     const int32_t S = m->S, M = m->M;
     const int64_t K = jb->K;
     const uint64_t i = (uint64_t)(jb->first + li);
-    int32_t x[64];
-    double a[256], cum[256];
+    int32_t x[ORACLE_SMAX];
+    static __thread double a[ORACLE_MMAX], cum[ORACLE_MMAX];
     for (int32_t s = 0; s < S; ++s) x[s] = m->x0[s];
     double t = 0.0;
     uint64_t step = 0;
@@ -227,7 +249,7 @@ static void simulate_instance(const job_t* jb, int64_t li) {
         for (int32_t j = 0; j < M; ++j) {
             uint64_t h = 1;
             for (int32_t e = 0; e < m->n_react[j]; ++e)
-                h *= binom(x[m->react_s[j * 4 + e]], m->react_r[j * 4 + e]);
+                h *= binom(x[m->react_s[j * ORACLE_RMAX + e]], m->react_r[j * ORACLE_RMAX + e]);
             a[j] = propensity(m, j, x, h);
         }
         /* a0 as a left-to-right running sum (R5) */
@@ -256,11 +278,25 @@ static void simulate_instance(const job_t* jb, int64_t li) {
         if (js < 0) for (int32_t j = M - 1; j >= 0; --j) if (a[j] > 0.0) { js = j; break; }
         /* multiset rewrite: x += nu_{j*} */
         for (int32_t s = 0; s < S; ++s) x[s] += m->delta[js * S + s];
+        /* reading R20: a creation fills the first free slot of its pool; a destruction moves the
+         * rest of the dissolved compartment to the context (or removes it) */
+        if (m->place_off)
+            for (int32_t p = m->place_off[js]; p < m->place_off[js + 1]; ++p)
+                if (x[m->place_alive[p]] == 0) {
+                    for (int32_t e = m->add_off[p]; e < m->add_off[p + 1]; ++e) x[m->add_s[e]] += m->add_n[e];
+                    break;
+                }
+        if (m->xfer_off)
+            for (int32_t e = m->xfer_off[js]; e < m->xfer_off[js + 1]; ++e) {
+                if (m->xfer_dst[e] >= 0) x[m->xfer_dst[e]] += x[m->xfer_src[e]];
+                x[m->xfer_src[e]] = 0;
+            }
         t = t_next;
         step += 1;
         reactions += 1;
         int over = 0;
         for (int32_t s = 0; s < S; ++s) if (x[s] > m->x_cap) over = 1;
+        if (m->sentinel >= 0 && x[m->sentinel] > 0) over = 1;
         if (over) {                           /* R9: freeze, remaining samples missing */
             flag = ORACLE_FLAG_OVERFLOWED;
             for (; k <= K; ++k) emit_missing(jb, li, k);
@@ -282,7 +318,7 @@ static void* worker(void* arg) {
 int oracle_simulate(const oracle_model* m, int64_t first, int64_t count, int64_t K, double dt,
                     uint64_t seed, int32_t nthreads, int32_t* raw, uint8_t* flags,
                     int64_t* reactions) {
-    if (!m || m->S <= 0 || m->S > 64 || m->M < 0 || m->M > 256 || count < 0 || K < 0 || !(dt > 0))
+    if (!m || m->S <= 0 || m->S > ORACLE_SMAX || m->M < 0 || m->M > ORACLE_MMAX || count < 0 || K < 0 || !(dt > 0))
         return -1;
     pthread_once(&cwclog_once, cwclog_init);
     if (nthreads < 1) nthreads = 1;
@@ -306,7 +342,7 @@ void oracle_propensities(const oracle_model* m, const int32_t* x, double* a, dou
     for (int32_t j = 0; j < m->M; ++j) {
         uint64_t h = 1;
         for (int32_t e = 0; e < m->n_react[j]; ++e)
-            h *= binom(x[m->react_s[j * 4 + e]], m->react_r[j * 4 + e]);
+            h *= binom(x[m->react_s[j * ORACLE_RMAX + e]], m->react_r[j * ORACLE_RMAX + e]);
         a[j] = propensity(m, j, x, h);
         c = c + a[j];
         cum[j] = c;

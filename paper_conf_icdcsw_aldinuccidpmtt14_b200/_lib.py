@@ -36,7 +36,13 @@ class ModelInfo(ctypes.Structure):
                 ("n_reactants", P(c_i32)), ("reactant_species", P(c_i32)), ("reactant_order", P(c_i32)),
                 ("delta", P(c_i32)), ("rule_of", P(c_i32)), ("x_cap", c_i64), ("x_cap_max", c_i64),
                 ("hist_bins", c_i32), ("hist_lo", P(c_i64)), ("hist_width", P(c_i64)),
-                ("law", P(c_i32)), ("law_species", P(c_i32)), ("law_K", P(c_dbl)), ("law_n", P(c_i32))]
+                ("law", P(c_i32)), ("law_species", P(c_i32)), ("law_K", P(c_dbl)), ("law_n", P(c_i32)),
+                ("gate_species", P(c_i32)), ("gate_kind", P(c_i32)), ("place_off", P(c_i32)),
+                ("place_alive", P(c_i32)), ("add_off", P(c_i32)), ("add_species", P(c_i32)),
+                ("add_count", P(c_i32)), ("xfer_off", P(c_i32)), ("xfer_src", P(c_i32)), ("xfer_dst", P(c_i32)),
+                ("sentinel", c_i32), ("flag", P(ctypes.c_uint8))]
+
+MAX_REACTANTS = 8  # CWC_MAX_REACTANTS
 
 
 class Stats(ctypes.Structure):

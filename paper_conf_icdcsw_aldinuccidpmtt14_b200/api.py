@@ -65,7 +65,7 @@ class Model:
                  quantiles: Optional[Sequence[float]] = None, raw_samples: bool = True,
                  quantum_samples: int = 0, block_threads: Optional[int] = None, refill: bool = True,
                  blocks_per_sm: int = 0, device: Optional[int] = None, period_species=None,
-                 period_lo: int = 0, period_hi: int = 1, period_window: int = 1, **options):
+                 period_lo: int = 0, period_hi: int = 1, period_window: int = 1, capacity=None, **options):
         sp = (ctypes.c_char_p * len(species))(*[s.encode() for s in species])
         rl = (ctypes.c_char_p * max(len(rules), 1))(*[r.encode() for r in rules])
         rt = (ctypes.c_double * max(len(rates), 1))(*[float(k) for k in rates])
@@ -73,6 +73,8 @@ class Model:
         check(lib.cwc_model_load(ctypes.byref(h), len(species), sp, len(rules), rl, rt, initial_term.encode()))
         self._h = h
         self._info_cache = None
+        for label, c in dict(capacity or {}).items():   # re-flattens: before species options (R20)
+            self.set_option(f"capacity.{label}", int(c))
         if x_cap is not None:
             self.set_option("x_cap", int(x_cap))
         if hist_bins is not None:
@@ -111,6 +113,8 @@ class Model:
         """Load a workloads.ModelDef-like object (species, rules, rates, initial_term, x_cap)."""
         if getattr(mdef, "x_cap", None) is not None and "x_cap" not in kw:
             kw["x_cap"] = mdef.x_cap
+        if getattr(mdef, "capacity", None) and "capacity" not in kw:
+            kw["capacity"] = dict(mdef.capacity)
         return cls(mdef.species, mdef.rules, mdef.rates, mdef.initial_term, **kw)
 
     def close(self):
@@ -142,12 +146,13 @@ class Model:
             mi = _lib.ModelInfo()
             check(lib.cwc_model_info(self._h, ctypes.byref(mi)))
             S, M = mi.n_species, mi.n_reactions
+            R = _lib.MAX_REACTANTS
             nre = [mi.n_reactants[j] for j in range(M)]
             self._info_cache = dict(
                 names=[mi.species_names[s].decode() for s in range(S)],
                 x0=[mi.x0[s] for s in range(S)],
                 rates=[mi.rates[j] for j in range(M)],
-                reactants=[[(mi.reactant_species[j * 4 + e], mi.reactant_order[j * 4 + e]) for e in range(nre[j])]
+                reactants=[[(mi.reactant_species[j * R + e], mi.reactant_order[j * R + e]) for e in range(nre[j])]
                            for j in range(M)],
                 delta=[[mi.delta[j * S + s] for s in range(S)] for j in range(M)],
                 rule_of=[mi.rule_of[j] for j in range(M)],
@@ -155,6 +160,14 @@ class Model:
                 hist_lo=[mi.hist_lo[s] for s in range(S)], hist_width=[mi.hist_width[s] for s in range(S)],
                 law=[mi.law[j] for j in range(M)], law_species=[mi.law_species[j] for j in range(M)],
                 law_K=[mi.law_K[j] for j in range(M)], law_n=[mi.law_n[j] for j in range(M)],
+                # reading R20 (dynamic compartments)
+                gate_species=[mi.gate_species[j] for j in range(M)], gate_kind=[mi.gate_kind[j] for j in range(M)],
+                place=[[(mi.place_alive[p], [(mi.add_species[e], mi.add_count[e])
+                                              for e in range(mi.add_off[p], mi.add_off[p + 1])])
+                        for p in range(mi.place_off[j], mi.place_off[j + 1])] for j in range(M)],
+                transfer=[[(mi.xfer_src[e], mi.xfer_dst[e]) for e in range(mi.xfer_off[j], mi.xfer_off[j + 1])]
+                          for j in range(M)],
+                sentinel=mi.sentinel, flag=[bool(mi.flag[s]) for s in range(S)],
             )
         return self._info_cache
 

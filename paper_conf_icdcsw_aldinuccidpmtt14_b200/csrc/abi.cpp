@@ -2,6 +2,7 @@
 // handling and exception -> status translation; the work is in compiler.cpp / runtime.cpp.
 #include <cmath>
 #include <cstring>
+#include <memory>
 #include <new>
 #include <string>
 
@@ -44,18 +45,58 @@ void refresh_info(cwc_model* m) {
     const int S = fm.S(), M = fm.M();
     m->name_ptrs.clear();
     for (auto& n : fm.names) m->name_ptrs.push_back(n.c_str());
+    const int R = CWC_MAX_REACTANTS;
     m->info_nreact.assign(M, 0);
-    m->info_rspecies.assign((size_t)M * 4, 0);
-    m->info_rorder.assign((size_t)M * 4, 0);
+    m->info_rspecies.assign((size_t)M * R, 0);
+    m->info_rorder.assign((size_t)M * R, 0);
     m->info_delta.assign((size_t)M * S, 0);
+    m->info_place_off.assign(1, 0);
+    m->info_add_off.assign(1, 0);
+    m->info_xfer_off.assign(1, 0);
+    m->info_place_alive.clear();
+    m->info_add_s.clear();
+    m->info_add_n.clear();
+    m->info_xfer_src.clear();
+    m->info_xfer_dst.clear();
     for (int j = 0; j < M; ++j) {
         m->info_nreact[j] = (int32_t)fm.reactants[j].size();
         for (size_t e = 0; e < fm.reactants[j].size(); ++e) {
-            m->info_rspecies[j * 4 + e] = fm.reactants[j][e].species;
-            m->info_rorder[j * 4 + e] = fm.reactants[j][e].order;
+            m->info_rspecies[j * R + e] = fm.reactants[j][e].species;
+            m->info_rorder[j * R + e] = fm.reactants[j][e].order;
         }
         for (int s = 0; s < S; ++s) m->info_delta[(size_t)j * S + s] = fm.delta[j][s];
+        for (const auto& ps : fm.place[j]) {
+            m->info_place_alive.push_back(ps.alive);
+            for (const auto& a : ps.adds) {
+                m->info_add_s.push_back(a.first);
+                m->info_add_n.push_back(a.second);
+            }
+            m->info_add_off.push_back((int32_t)m->info_add_s.size());
+        }
+        m->info_place_off.push_back((int32_t)m->info_place_alive.size());
+        for (const auto& x : fm.transfer[j]) {
+            m->info_xfer_src.push_back(x.first);
+            m->info_xfer_dst.push_back(x.second);
+        }
+        m->info_xfer_off.push_back((int32_t)m->info_xfer_src.size());
     }
+}
+
+// (Re)flatten the stored load inputs and reset every species-indexed option.
+void flatten_into(cwc_model* m) {
+    cwc::FlatModel fm = cwc::compile_model(m->in_alphabet, m->in_rules, m->in_rates, m->in_term, m->capacity);
+    for (const auto& rl : fm.reactants)
+        if ((int)rl.size() > CWC_MAX_REACTANTS)
+            fail(CWC_E_UNSUPPORTED, "a flat reaction has more than CWC_MAX_REACTANTS reactant species");
+    for (int32_t v : fm.x0)
+        if (v > fm.x_cap_max) fail(CWC_E_INVALID, "initial count above the largest exact cap");
+    m->fm = std::move(fm);
+    m->x_cap = m->fm.x_cap_max;
+    m->hist_lo.assign(m->fm.S(), 0);
+    m->hist_width.assign(m->fm.S(), 1);
+    m->period_species = -1;
+    m->compiled_key.clear();
+    refresh_info(m);
 }
 
 int species_index(const cwc_model* m, const std::string& name) {
@@ -91,19 +132,13 @@ cwc_status cwc_model_load(cwc_model_t* out, int32_t n_species, const char* const
             rs.emplace_back(rules[i]);
             ks.push_back(rates[i]);
         }
-        cwc::FlatModel fm = cwc::compile_model(alpha, rs, ks, initial_term);
-        cwc_model* m = new cwc_model();
-        m->fm = std::move(fm);
-        m->x_cap = m->fm.x_cap_max;
-        for (int32_t v : m->fm.x0)
-            if (v > m->x_cap) {
-                delete m;
-                fail(CWC_E_INVALID, "initial count above the largest exact cap");
-            }
-        m->hist_lo.assign(m->fm.S(), 0);
-        m->hist_width.assign(m->fm.S(), 1);
-        refresh_info(m);
-        *out = m;
+        std::unique_ptr<cwc_model> m(new cwc_model());
+        m->in_alphabet = alpha;
+        m->in_rules = rs;
+        m->in_rates = ks;
+        m->in_term = initial_term;
+        flatten_into(m.get());
+        *out = m.release();
     });
 }
 
@@ -137,6 +172,18 @@ cwc_status cwc_model_info(cwc_model_t m, cwc_model_info_t* out) {
         out->law_species = m->fm.law_species.data();
         out->law_K = m->fm.law_K.data();
         out->law_n = m->fm.law_n.data();
+        out->gate_species = m->fm.gate_species.data();
+        out->gate_kind = m->fm.gate_kind.data();
+        out->place_off = m->info_place_off.data();
+        out->place_alive = m->info_place_alive.data();
+        out->add_off = m->info_add_off.data();
+        out->add_species = m->info_add_s.data();
+        out->add_count = m->info_add_n.data();
+        out->xfer_off = m->info_xfer_off.data();
+        out->xfer_src = m->info_xfer_src.data();
+        out->xfer_dst = m->info_xfer_dst.data();
+        out->sentinel = m->fm.sentinel;
+        out->flag = m->fm.flag.data();
     });
 }
 
@@ -144,7 +191,19 @@ cwc_status cwc_set_option_i64(cwc_model_t m, const char* key, int64_t v) {
     return guard([&] {
         need(m && key, "NULL argument");
         std::string k(key);
-        if (k == "x_cap") {
+        if (k.rfind("capacity.", 0) == 0) {
+            need(v >= 1 && v <= 4096, "capacity outside [1, 4096]");
+            const std::string label = k.substr(9);
+            const auto old = m->capacity;
+            m->capacity[label] = v;
+            try {
+                flatten_into(m);
+            } catch (...) {
+                m->capacity = old;
+                flatten_into(m);
+                throw;
+            }
+        } else if (k == "x_cap") {
             need(v >= 1 && v <= m->fm.x_cap_max, "x_cap outside [1, x_cap_max]");
             for (int32_t x : m->fm.x0) need(x <= v, "x_cap below an initial count");
             m->x_cap = v;

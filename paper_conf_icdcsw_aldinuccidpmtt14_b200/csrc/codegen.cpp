@@ -23,6 +23,7 @@ std::string hexd(double v) {
 
 std::string generate_model_section(const FlatModel& fm, const KernelConfig& cfg) {
     const int S = fm.S(), M = fm.M();
+    auto is_flag = [&](int sp) { return fm.flag.size() == (size_t)S && fm.flag[sp]; };
     std::ostringstream o;
     o << "// ---- generated model section: " << S << " species, " << M << " flat reactions\n";
     o << "#define CWC_S " << S << "\n#define CWC_M " << (M > 0 ? M : 1) << "\n#define CWC_B " << cfg.hist_bins
@@ -56,7 +57,8 @@ std::string generate_model_section(const FlatModel& fm, const KernelConfig& cfg)
     // per-(species, order) binomial factors, shared between reactions
     std::vector<std::vector<bool>> need(S, std::vector<bool>(4, false));
     for (int j = 0; j < M; ++j) {
-        for (const Reactant& r : fm.reactants[j]) need[r.species][r.order] = true;
+        for (const Reactant& r : fm.reactants[j])
+            if (!is_flag(r.species)) need[r.species][r.order] = true;
         if (fm.law[j] != LAW_MASS_ACTION) need[fm.law_species[j]][1] = true;
     }
     for (int s = 0; s < S; ++s) {
@@ -71,16 +73,28 @@ std::string generate_model_section(const FlatModel& fm, const KernelConfig& cfg)
     if (M == 0) o << "    a[0] = 0.0;\n";
     for (int j = 0; j < M; ++j) {
         std::string h;
+        // occupancy flags (R20) are 0/1: k * h * flag == (flag ? k * h : 0.0) exactly, so they
+        // select instead of multiplying
+        std::string flags;
+        for (const Reactant& r : fm.reactants[j])
+            if (is_flag(r.species)) flags += std::string(flags.empty() ? "" : " && ") + "x[" + std::to_string(r.species) + "] != 0";
         for (const Reactant& r : fm.reactants[j]) {
+            if (is_flag(r.species)) continue;
             std::string f = "f" + std::to_string(r.species) + "_" + std::to_string(r.order);
             h = h.empty() ? f : "__dmul_rn(" + h + ", " + f + ")";
         }
+        // reading R20: a gated reaction (creation / pool full) is enabled while x_g >= 1 / x_g == 0
+        std::string gate = flags;
+        if (!fm.gate_species.empty() && fm.gate_species[j] >= 0)
+            gate += std::string(gate.empty() ? "" : " && ") + "x[" + std::to_string(fm.gate_species[j]) +
+                    (fm.gate_kind[j] == GATE_POSITIVE ? "] >= 1" : "] == 0");
         if (fm.law[j] == LAW_MASS_ACTION) {
-            o << "    a[" << j << "] = "
-              << (h.empty() ? hexd(fm.rates[j]) : "__dmul_rn(" + hexd(fm.rates[j]) + ", " + h + ")")
-              << ";  // rule " << fm.rule_of[j] << "\n";
+            std::string e = h.empty() ? hexd(fm.rates[j]) : "__dmul_rn(" + hexd(fm.rates[j]) + ", " + h + ")";
+            if (!gate.empty()) e = "(" + gate + ") ? " + e + " : 0.0";
+            o << "    a[" << j << "] = " << e << ";  // rule " << fm.rule_of[j] << "\n";
             continue;
         }
+        if (!gate.empty()) h = h.empty() ? "((" + gate + ") ? 1.0 : 0.0)" : "__dmul_rn(" + h + ", (" + gate + ") ? 1.0 : 0.0)";
         // functional rate law (R16'): k*X/(K+X), k*X^n/(K^n+X^n) or k*K^n/(K^n+X^n), only when the
         // lhs is available; powers are left-to-right products, K^n computed on the host the same way
         const std::string X = "f" + std::to_string(fm.law_species[j]) + "_1";
@@ -129,11 +143,40 @@ std::string generate_model_section(const FlatModel& fm, const KernelConfig& cfg)
                 maxabs = std::max(maxabs, std::abs(fm.delta[j][s]));
                 if (fm.delta[j][s] > 0) inc[s] = true;
             }
+    // reading R20: creations (first free slot of a pool) and destructions (moves of the rest)
+    // depend on the state, so they are applied by rule index after the delta
+    std::vector<int> special;
+    for (int j = 0; j < M; ++j)
+        if ((!fm.place.empty() && !fm.place[j].empty()) || (!fm.transfer.empty() && !fm.transfer[j].empty())) {
+            special.push_back(j);
+            for (const auto& ps : fm.place[j])
+                for (const auto& a : ps.adds) inc[a.first] = true;
+            for (const auto& x : fm.transfer[j])
+                if (x.second >= 0) inc[x.second] = true;
+        }
+    std::string special_code;
+    for (int j : special) {
+        std::ostringstream so;
+        so << "    if (j == " << j << ") {\n";
+        bool first = true;
+        for (const auto& ps : fm.place[j]) {
+            so << "        " << (first ? "if" : "else if") << " (x[" << ps.alive << "] == 0) {";
+            for (const auto& a : ps.adds) so << " x[" << a.first << "] += " << a.second << ";";
+            so << " }\n";
+            first = false;
+        }
+        for (const auto& x : fm.transfer[j]) {
+            if (x.second >= 0) so << "        x[" << x.second << "] += x[" << x.first << "];\n";
+            so << "        x[" << x.first << "] = 0;\n";
+        }
+        so << "    }\n";
+        special_code += so.str();
+    }
     const bool table = (cfg.delta_table == 1 || (cfg.delta_table < 0 && pairs > 2 * S)) && maxabs <= 127 && M > 0;
     // fast-path rewrite straight from the selection predicates p_i = (cum_i <= target), which are
     // monotone (cum is non-decreasing), so p_i = [i < j*] and the telescoping sum
     // nu_0 + sum_{i<M-1} (nu_{i+1} - nu_i) p_i = nu_{j*} needs no rule index at all
-    const bool telescope = !table && M > 1 && (cfg.delta_table == 2 || cfg.delta_table < 0);
+    const bool telescope = !table && M > 1 && special.empty() && (cfg.delta_table == 2 || cfg.delta_table < 0);
     if (telescope) {
         o << "#define CWC_TELESCOPE 1\n";
         o << "__device__ __forceinline__ bool cwc_apply_p(const bool (&p)[CWC_M], int (&x)[CWC_S]) {\n";
@@ -202,9 +245,12 @@ std::string generate_model_section(const FlatModel& fm, const KernelConfig& cfg)
             if (chain != "0") o << "    x[" << s << "] += " << chain << ";\n";
         }
     }
+    o << special_code;
     o << "    bool over = false;\n";
     for (int s = 0; s < S; ++s)
-        if (inc[s]) o << "    over |= x[" << s << "] > CWC_X_CAP;\n";
+        if (inc[s] && !(fm.flag.size() == (size_t)S && fm.flag[s]) && s != fm.sentinel)
+            o << "    over |= x[" << s << "] > CWC_X_CAP;\n";
+    if (fm.sentinel >= 0) o << "    over |= x[" << fm.sentinel << "] > 0;  // a pool was full (R20)\n";
     o << "    return over;\n}\n\n";
 
     // histogram bins: 0 underflow, 1..B, B+1 overflow (R11)

@@ -116,8 +116,9 @@ class Parser {
     // A sequence of atoms / n*A / '.' / variable; compartments only where allowed.
     // Stops at End, Arrow, or one of the stop symbols.
     // comps: 0 = compartment is a parse error, 1 = unsupported, 2 = allowed.
+    // vars (a rule's right-hand side at rule level, reading R20): the released variables.
     void sequence(const char* stops, int comps_policy, Counts& atoms, std::string* var,
-                  std::vector<Comp>* comps, std::vector<PComp>* pcomps) {
+                  std::vector<Comp>* comps, std::vector<PComp>* pcomps, std::vector<std::string>* vars = nullptr) {
         while (true) {
             const Token& t = peek();
             if (t.kind == Tok::End || t.kind == Tok::Arrow) return;
@@ -132,6 +133,12 @@ class Parser {
                 atoms[atom(tk.text)] += 1;
             } else if (tk.kind == Tok::Var) {
                 if (!pattern_) throw Error(CWC_E_PARSE, "variable " + tk.text + " in a term");
+                if (vars) {
+                    if (std::find(vars->begin(), vars->end(), tk.text) != vars->end())
+                        throw Error(CWC_E_UNSUPPORTED, "variable " + tk.text + " released twice: '" + src_ + "'");
+                    vars->push_back(tk.text);
+                    continue;
+                }
                 if (!var) throw Error(CWC_E_UNSUPPORTED, "variable at rule level: '" + src_ + "'");
                 if (!var->empty()) throw Error(CWC_E_UNSUPPORTED, "two variables in one multiset: '" + src_ + "'");
                 *var = tk.text;
@@ -190,6 +197,11 @@ struct Rule {
     int law_atom = -1;
     double law_K = 0.0;
     int32_t law_n = 1;
+    // reading R20: per lhs pattern compartment the rhs compartment it persists as (-1:
+    // destroyed), the created rhs compartment (-1: none), the released rule-level variables
+    std::vector<int> keep;
+    int create = -1;
+    std::vector<std::string> release;
 };
 
 bool valid_ident(const std::string& s) {
@@ -265,25 +277,49 @@ Rule parse_rule(const std::string& text, const std::unordered_map<std::string, i
     for (int k = 0; k < 2; ++k) {
         Parser p(sides[k], atoms, true);
         pats[k]->atoms.assign(atoms.size(), 0);
-        p.sequence("", 2, pats[k]->atoms, nullptr, nullptr, &pats[k]->comps);
+        p.sequence("", 2, pats[k]->atoms, nullptr, nullptr, &pats[k]->comps, k == 1 ? &r.release : nullptr);
         if (!p.at_end()) throw Error(CWC_E_PARSE, "trailing input in '" + sides[k] + "'");
     }
-    // Static structure: the k-th rhs compartment is the k-th lhs compartment, same label and
-    // variables; both variables present (open patterns).
-    if (r.lhs.comps.size() != r.rhs.comps.size())
-        throw Error(CWC_E_UNSUPPORTED, "compartment creation/destruction: '" + text + "'");
+    // Structure (readings R15, R20): an rhs compartment carrying the variables of an lhs pattern
+    // compartment is that compartment (same label); an rhs compartment without variables is
+    // created (at most one per rule); an lhs compartment that does not reappear is destroyed and
+    // its variables may be released at rule level.  Pattern compartments are open (both
+    // variables present).
     std::set<std::string> seen;
-    for (size_t c = 0; c < r.lhs.comps.size(); ++c) {
-        const PComp &a = r.lhs.comps[c], &b = r.rhs.comps[c];
-        if (a.label != b.label) throw Error(CWC_E_UNSUPPORTED, "relabelling a compartment: '" + text + "'");
+    for (const PComp& a : r.lhs.comps) {
         if (a.wvar.empty() || a.cvar.empty())
             throw Error(CWC_E_UNSUPPORTED, "pattern compartment without $wrap/$content variables: '" + text + "'");
-        if (a.wvar != b.wvar || a.cvar != b.cvar)
-            throw Error(CWC_E_UNSUPPORTED, "variables moved between compartments: '" + text + "'");
-        for (const std::string* v : {&a.wvar, &a.cvar}) {
+        for (const std::string* v : {&a.wvar, &a.cvar})
             if (!seen.insert(*v).second) throw Error(CWC_E_UNSUPPORTED, "variable " + *v + " used twice: '" + text + "'");
-        }
     }
+    r.keep.assign(r.lhs.comps.size(), -1);
+    for (size_t bi = 0; bi < r.rhs.comps.size(); ++bi) {
+        const PComp& b = r.rhs.comps[bi];
+        if (b.wvar.empty() && b.cvar.empty()) {
+            if (r.create >= 0) throw Error(CWC_E_UNSUPPORTED, "more than one compartment created: '" + text + "'");
+            r.create = (int)bi;
+            continue;
+        }
+        int match = -1;
+        for (size_t ai = 0; ai < r.lhs.comps.size(); ++ai)
+            if (r.lhs.comps[ai].wvar == b.wvar && r.lhs.comps[ai].cvar == b.cvar) {
+                match = (int)ai;
+                break;
+            }
+        if (match < 0 || r.keep[match] >= 0)
+            throw Error(CWC_E_UNSUPPORTED, "variables moved between compartments: '" + text + "'");
+        if (r.lhs.comps[match].label != b.label) throw Error(CWC_E_UNSUPPORTED, "relabelling a compartment: '" + text + "'");
+        r.keep[match] = (int)bi;
+    }
+    std::set<std::string> gone;
+    for (size_t ai = 0; ai < r.lhs.comps.size(); ++ai)
+        if (r.keep[ai] < 0) {
+            gone.insert(r.lhs.comps[ai].wvar);
+            gone.insert(r.lhs.comps[ai].cvar);
+        }
+    for (const std::string& v : r.release)
+        if (!gone.count(v))
+            throw Error(CWC_E_UNSUPPORTED, "variable " + v + " released but its compartment is not destroyed: '" + text + "'");
     return r;
 }
 
@@ -294,26 +330,88 @@ struct Region {
     bool wrap;
     Counts atoms;
     std::vector<int> child_content, child_wrap;
+    int pool = -1, slot = -1;  // the pool slot this region belongs to (reading R20)
 };
 
-int add_content(std::vector<Region>& regs, const Node& node, const std::string& name, const std::string& owner) {
-    int idx = (int)regs.size();
-    regs.push_back(Region{name, owner, false, node.atoms, {}, {}});
-    std::map<std::string, int> total, seen;
-    for (const Comp& c : node.comps) total[c.label]++;
-    for (const Comp& c : node.comps) {
-        std::string seg = c.label;
-        if (total[c.label] > 1) seg += "#" + std::to_string(seen[c.label]);
-        seen[c.label]++;
-        std::string path = name.empty() ? seg : name + "/" + seg;
-        int w = (int)regs.size();
-        regs.push_back(Region{path + ".wrap", c.label, true, c.wrap, {}, {}});
-        int ci = add_content(regs, *c.content, path, c.label);
-        regs[idx].child_wrap.push_back(w);
-        regs[idx].child_content.push_back(ci);
+// Reading R20: the slots for the dynamic compartments of one label in one content region.
+struct Pool {
+    int parent;
+    std::string label;
+    std::vector<std::pair<int, int>> slots;  // (wrap region, content region)
+    int occupied;                             // slots 0..occupied-1 filled by the initial term
+};
+
+struct RegionBuilder {
+    std::vector<Region>& regs;
+    std::vector<Pool>& pools;
+    const std::set<std::string>& dynamic;
+    const std::set<std::pair<std::string, std::string>>& creators;  // (context label, created label)
+    const std::map<std::string, int64_t>& capacity;
+
+    // Pre-order: the content region, each static child (wrap, content, recursively), then the
+    // pools of dynamic children in label order, slot by slot (wrap, content).
+    int add_content(const Node& node, const std::string& name, const std::string& owner) {
+        int idx = (int)regs.size();
+        regs.push_back(Region{name, owner, false, node.atoms, {}, {}});
+        std::map<std::string, int> total, seen;
+        for (const Comp& c : node.comps)
+            if (!dynamic.count(c.label)) total[c.label]++;
+        std::map<std::string, std::vector<const Comp*>> dyn;
+        for (const Comp& c : node.comps) {
+            if (dynamic.count(c.label)) {
+                if (!c.content->comps.empty())
+                    throw Error(CWC_E_UNSUPPORTED, "dynamic compartment '" + c.label + "' with nested compartments");
+                dyn[c.label].push_back(&c);
+                continue;
+            }
+            std::string seg = c.label;
+            if (total[c.label] > 1) seg += "#" + std::to_string(seen[c.label]);
+            seen[c.label]++;
+            std::string path = name.empty() ? seg : name + "/" + seg;
+            int w = (int)regs.size();
+            regs.push_back(Region{path + ".wrap", c.label, true, c.wrap, {}, {}});
+            int ci = add_content(*c.content, path, c.label);
+            regs[idx].child_wrap.push_back(w);
+            regs[idx].child_content.push_back(ci);
+        }
+        std::set<std::string> labels;
+        for (auto& kv : dyn) labels.insert(kv.first);
+        for (auto& cr : creators)
+            if (cr.first == owner) labels.insert(cr.second);
+        const size_t A = node.atoms.size();
+        for (const std::string& l : labels) {
+            const std::vector<const Comp*>& init = dyn[l];
+            auto it = capacity.find(l);
+            const int64_t cap = it == capacity.end() ? kDefaultCapacity : it->second;
+            if (cap < 1 || cap > 4096 || (int64_t)init.size() > cap)
+                throw Error(CWC_E_INVALID, "capacity of '" + l + "' must be in [1, 4096] and hold the initial compartments");
+            const int pid = (int)pools.size();
+            pools.push_back(Pool{idx, l, {}, (int)init.size()});
+            for (int k = 0; k < (int)cap; ++k) {
+                std::string seg = l + "[" + std::to_string(k) + "]";
+                std::string path = name.empty() ? seg : name + "/" + seg;
+                Counts w(A, 0), ct(A, 0);
+                if (k < (int)init.size()) {
+                    w = init[k]->wrap;
+                    ct = init[k]->content->atoms;
+                }
+                int wi = (int)regs.size();
+                regs.push_back(Region{path + ".wrap", l, true, w, {}, {}, pid, k});
+                int ci = (int)regs.size();
+                regs.push_back(Region{path, l, false, ct, {}, {}, pid, k});
+                regs[idx].child_wrap.push_back(wi);
+                regs[idx].child_content.push_back(ci);
+                pools[pid].slots.push_back({wi, ci});
+            }
+        }
+        return idx;
     }
-    return idx;
-}
+};
+
+struct Destroyed {
+    int wrap, content;
+    bool rel_wrap, rel_content;
+};
 
 struct RawReaction {
     int rule;
@@ -321,6 +419,13 @@ struct RawReaction {
     int ctx;  // context region (where a rate law's species is read)
     std::map<std::pair<int, int>, int64_t> react;   // (region, atom) -> order
     std::map<std::pair<int, int>, int64_t> delta;   // (region, atom) -> net change (may be 0)
+    // reading R20
+    std::pair<int, int> gate{-1, -1};
+    int gate_kind = GATE_NONE;
+    int place_pool = -1;                             // creation into this pool
+    const PComp* created = nullptr;
+    std::vector<Destroyed> destroyed;
+    std::vector<std::pair<std::pair<int, int>, std::pair<int, int>>> xfer;  // src -> dst ((-1,-1) removed)
 };
 
 // Enumerate injective, label-matching assignments of pattern compartments to children, in
@@ -371,7 +476,8 @@ int64_t max_exact_cap(const std::vector<std::vector<Reactant>>& reactants, int64
 }
 
 FlatModel compile_model(const std::vector<std::string>& alphabet, const std::vector<std::string>& rules,
-                        const std::vector<double>& rates, const std::string& initial_term) {
+                        const std::vector<double>& rates, const std::string& initial_term,
+                        const std::map<std::string, int64_t>& capacity) {
     if (alphabet.empty()) throw Error(CWC_E_INVALID, "empty alphabet");
     if (rules.size() != rates.size()) throw Error(CWC_E_INVALID, "one rate per rule");
     std::unordered_map<std::string, int> atoms;
@@ -379,7 +485,7 @@ FlatModel compile_model(const std::vector<std::string>& alphabet, const std::vec
         if (!valid_ident(alphabet[i]) || alphabet[i] == "top") throw Error(CWC_E_INVALID, "bad atom name '" + alphabet[i] + "'");
         if (!atoms.emplace(alphabet[i], (int)i).second) throw Error(CWC_E_INVALID, "duplicate atom '" + alphabet[i] + "'");
     }
-    const size_t A = alphabet.size();
+    const int A = (int)alphabet.size();
 
     Node top{Counts(A, 0), {}};
     {
@@ -390,10 +496,38 @@ FlatModel compile_model(const std::vector<std::string>& alphabet, const std::vec
     std::vector<Rule> parsed;
     for (size_t i = 0; i < rules.size(); ++i) parsed.push_back(parse_rule(rules[i], atoms, rates[i]));
 
-    std::vector<Region> regs;
-    add_content(regs, top, "", "top");
+    // Reading R20: a label is dynamic when a rule creates or destroys a compartment of it.
+    std::set<std::string> dynamic;
+    std::set<std::pair<std::string, std::string>> creators;
+    for (const Rule& r : parsed) {
+        if (r.create >= 0) {
+            dynamic.insert(r.rhs.comps[r.create].label);
+            creators.insert({r.label, r.rhs.comps[r.create].label});
+        }
+        for (size_t a = 0; a < r.lhs.comps.size(); ++a)
+            if (r.keep[a] < 0) dynamic.insert(r.lhs.comps[a].label);
+    }
+    for (auto& cr : creators)
+        if (dynamic.count(cr.first))
+            throw Error(CWC_E_UNSUPPORTED, "compartment '" + cr.second + "' created inside dynamic compartment '" + cr.first + "'");
+    for (auto& kv : capacity)
+        if (!dynamic.count(kv.first)) throw Error(CWC_E_INVALID, "capacity of '" + kv.first + "': not a dynamic compartment");
 
-    // Tree matching once: every (rule, context, assignment) is a flat reaction.
+    std::vector<Region> regs;
+    std::vector<Pool> pools;
+    RegionBuilder rb{regs, pools, dynamic, creators, capacity};
+    rb.add_content(top, "", "top");
+    std::map<std::pair<int, std::string>, int> pool_of;
+    for (size_t p = 0; p < pools.size(); ++p) pool_of[{pools[p].parent, pools[p].label}] = (int)p;
+    // pseudo-atoms of the flag species (ordered after the alphabet within a region)
+    std::vector<std::string> dyn_labels(dynamic.begin(), dynamic.end());  // sorted
+    const int ALIVE = A, FULL = A + 1 + (int)dyn_labels.size();
+    auto FREE = [&](const std::string& l) {
+        return A + 1 + (int)(std::lower_bound(dyn_labels.begin(), dyn_labels.end(), l) - dyn_labels.begin());
+    };
+    auto alive_of = [&](int region) { return std::make_pair(pools[regs[region].pool].slots[regs[region].slot].second, ALIVE); };
+
+    // Tree matching once: every (rule, context, assignment) is a flat reaction (two for a creation).
     std::vector<RawReaction> raw;
     for (size_t ri = 0; ri < parsed.size(); ++ri) {
         const Rule& rule = parsed[ri];
@@ -405,42 +539,111 @@ FlatModel compile_model(const std::vector<std::string>& alphabet, const std::vec
             std::vector<bool> used(ctx.child_content.size(), false);
             assignments(regs, ctx, rule.lhs.comps, cur, used, found);
             for (const auto& asg : found) {
-                RawReaction rr{(int)ri, rule.rate, (int)ci, {}, {}};
-                auto add = [](std::map<std::pair<int, int>, int64_t>& m, int reg, const Counts& c, int64_t sign) {
+                RawReaction rr;
+                rr.rule = (int)ri;
+                rr.rate = rule.rate;
+                rr.ctx = (int)ci;
+                std::map<std::pair<int, int>, int64_t> prod;
+                auto add = [](std::map<std::pair<int, int>, int64_t>& m, int reg, const Counts& c) {
                     for (size_t a = 0; a < c.size(); ++a)
-                        if (c[a]) m[{reg, (int)a}] += sign * c[a];
+                        if (c[a]) m[{reg, (int)a}] += c[a];
                 };
-                add(rr.react, (int)ci, rule.lhs.atoms, 1);
-                add(rr.delta, (int)ci, rule.rhs.atoms, 1);
-                add(rr.delta, (int)ci, rule.lhs.atoms, -1);
+                add(rr.react, (int)ci, rule.lhs.atoms);
+                add(prod, (int)ci, rule.rhs.atoms);
+                if (ctx.pool >= 0) {  // inside a pool slot: only while it is occupied
+                    rr.react[alive_of((int)ci)] += 1;
+                    prod[alive_of((int)ci)] += 1;
+                }
                 for (size_t p = 0; p < asg.size(); ++p) {
                     int w = ctx.child_wrap[asg[p]], c = ctx.child_content[asg[p]];
-                    add(rr.react, w, rule.lhs.comps[p].wrap, 1);
-                    add(rr.react, c, rule.lhs.comps[p].content, 1);
-                    add(rr.delta, w, rule.rhs.comps[p].wrap, 1);
-                    add(rr.delta, c, rule.rhs.comps[p].content, 1);
-                    add(rr.delta, w, rule.lhs.comps[p].wrap, -1);
-                    add(rr.delta, c, rule.lhs.comps[p].content, -1);
+                    const PComp& pc = rule.lhs.comps[p];
+                    add(rr.react, w, pc.wrap);
+                    add(rr.react, c, pc.content);
+                    if (regs[c].pool >= 0) rr.react[alive_of(c)] += 1;
+                    if (rule.keep[p] >= 0) {
+                        const PComp& qc = rule.rhs.comps[rule.keep[p]];
+                        add(prod, w, qc.wrap);
+                        add(prod, c, qc.content);
+                        if (regs[c].pool >= 0) prod[alive_of(c)] += 1;
+                    } else {  // destroyed: the slot is freed, the rest moved or removed
+                        const Pool& pl = pools[regs[c].pool];
+                        prod[{pl.parent, FREE(pl.label)}] += 1;
+                        const bool rw = std::find(rule.release.begin(), rule.release.end(), pc.wvar) != rule.release.end();
+                        const bool rc = std::find(rule.release.begin(), rule.release.end(), pc.cvar) != rule.release.end();
+                        rr.destroyed.push_back(Destroyed{w, c, rw, rc});
+                    }
                 }
                 int64_t order = 0;
-                for (auto& kv : rr.react) order += kv.second;
+                for (auto& kv : rr.react)
+                    if (kv.first.second != ALIVE) order += kv.second;
                 if (order > 3) throw Error(CWC_E_UNSUPPORTED, "reaction order > 3 in rule " + std::to_string(ri));
+                for (auto& kv : prod) rr.delta[kv.first] += kv.second;
+                for (auto& kv : rr.react) rr.delta[kv.first] -= kv.second;
+                if (rule.create < 0) {
+                    raw.push_back(std::move(rr));
+                    continue;
+                }
+                // creation: into the lowest free slot of the pool, else the pool is full
+                const PComp& qc = rule.rhs.comps[rule.create];
+                const int pid = pool_of.at({(int)ci, qc.label});
+                const std::pair<int, int> fkey{(int)ci, FREE(qc.label)};
+                RawReaction full = rr;
+                rr.gate = fkey;
+                rr.gate_kind = GATE_POSITIVE;
+                rr.delta[fkey] -= 1;
+                rr.place_pool = pid;
+                rr.created = &qc;
+                full.gate = fkey;
+                full.gate_kind = GATE_ZERO;
+                full.delta.clear();
+                full.delta[{0, FULL}] = 1;
+                full.destroyed.clear();
                 raw.push_back(std::move(rr));
+                raw.push_back(std::move(full));
             }
         }
     }
 
-    // Species: every (region, atom) present initially or touched by a reaction; region
-    // pre-order, then alphabet order.
+    // Species: every (region, atom) present initially or touched by a reaction, the flags of
+    // every pool, "#full" when a pool can overflow; region pre-order, then alphabet order, then
+    // "#alive", "#free:<label>" (label order), "#full".
     std::set<std::pair<int, int>> used;
     for (size_t r = 0; r < regs.size(); ++r)
-        for (size_t a = 0; a < A; ++a)
-            if (regs[r].atoms[a] > 0) used.insert({(int)r, (int)a});
+        for (int a = 0; a < A; ++a)
+            if (regs[r].atoms[a] > 0) used.insert({(int)r, a});
+    for (const Pool& pl : pools) {
+        used.insert({pl.parent, FREE(pl.label)});
+        for (auto& sl : pl.slots) used.insert({sl.second, ALIVE});
+    }
+    bool has_full = false;
     for (const auto& rr : raw) {
         for (auto& kv : rr.react) used.insert(kv.first);
         for (auto& kv : rr.delta) used.insert(kv.first);
+        if (rr.gate.first >= 0) used.insert(rr.gate);
+        if (rr.gate_kind == GATE_ZERO) has_full = true;
+        if (rr.place_pool >= 0)
+            for (auto& sl : pools[rr.place_pool].slots)
+                for (int a = 0; a < A; ++a) {
+                    if (rr.created->wrap[a]) used.insert({sl.first, a});
+                    if (rr.created->content[a]) used.insert({sl.second, a});
+                }
         if (parsed[rr.rule].law != LAW_MASS_ACTION) used.insert({rr.ctx, parsed[rr.rule].law_atom});
     }
+    if (has_full) used.insert({0, FULL});
+    for (auto& rr : raw)
+        for (const Destroyed& d : rr.destroyed)
+            for (int k = 0; k < 2; ++k) {
+                const int reg = k == 0 ? d.wrap : d.content;
+                const bool rel = k == 0 ? d.rel_wrap : d.rel_content;
+                std::vector<std::pair<int, int>> srcs;
+                for (auto& ra : used)
+                    if (ra.first == reg && ra.second < A) srcs.push_back(ra);
+                for (auto& src : srcs) {
+                    std::pair<int, int> dst = rel ? std::make_pair(rr.ctx, src.second) : std::make_pair(-1, -1);
+                    rr.xfer.push_back({src, dst});
+                    if (rel) used.insert(dst);
+                }
+            }
     if (used.empty()) throw Error(CWC_E_INVALID, "model has no species");
 
     FlatModel fm;
@@ -450,16 +653,37 @@ FlatModel compile_model(const std::vector<std::string>& alphabet, const std::vec
     for (const auto& ra : used) {  // std::set order == (region, atom) lexicographic
         sidx[ra] = (int)fm.names.size();
         const Region& reg = regs[ra.first];
-        fm.names.push_back(reg.name.empty() ? alphabet[ra.second] : alphabet[ra.second] + "@" + reg.name);
-        int64_t v = reg.atoms[ra.second];
+        std::string atom;
+        int64_t v = 0;
+        if (ra.second < A) {
+            atom = alphabet[ra.second];
+            v = reg.atoms[ra.second];
+        } else if (ra.second == ALIVE) {
+            atom = "#alive";
+            v = reg.slot < pools[reg.pool].occupied ? 1 : 0;
+        } else if (ra.second == FULL) {
+            atom = "#full";
+        } else {
+            const std::string& l = dyn_labels[ra.second - A - 1];
+            atom = "#free:" + l;
+            const Pool& pl = pools[pool_of.at({ra.first, l})];
+            v = (int64_t)pl.slots.size() - pl.occupied;
+        }
+        fm.names.push_back(reg.name.empty() ? atom : atom + "@" + reg.name);
         if (v > (int64_t)INT32_MAX) throw Error(CWC_E_INVALID, "initial count too large");
         fm.x0.push_back((int32_t)v);
+        fm.flag.push_back(ra.second == ALIVE ? 1 : 0);
     }
+    fm.sentinel = has_full ? sidx[{0, FULL}] : -1;
     const int S = (int)fm.names.size();
+    std::vector<std::vector<Reactant>> cap_lists;
     for (const auto& rr : raw) {
-        std::vector<Reactant> rl;
+        std::vector<Reactant> rl, rl_cap;
         for (auto& kv : rr.react) rl.push_back(Reactant{sidx[kv.first], (int32_t)kv.second});
         std::sort(rl.begin(), rl.end(), [](const Reactant& a, const Reactant& b) { return a.species < b.species; });
+        for (const Reactant& e : rl)
+            if (!fm.flag[e.species]) rl_cap.push_back(e);
+        cap_lists.push_back(rl_cap);
         std::vector<int32_t> d(S, 0);
         for (auto& kv : rr.delta) d[sidx[kv.first]] += (int32_t)kv.second;
         fm.reactants.push_back(rl);
@@ -471,8 +695,30 @@ FlatModel compile_model(const std::vector<std::string>& alphabet, const std::vec
         fm.law_species.push_back(rule.law == LAW_MASS_ACTION ? -1 : sidx[{rr.ctx, rule.law_atom}]);
         fm.law_K.push_back(rule.law_K);
         fm.law_n.push_back(rule.law_n);
+        fm.gate_species.push_back(rr.gate.first >= 0 ? sidx[rr.gate] : -1);
+        fm.gate_kind.push_back(rr.gate_kind);
+        std::vector<FlatModel::PlaceSlot> place;
+        if (rr.place_pool >= 0)
+            for (auto& sl : pools[rr.place_pool].slots) {
+                FlatModel::PlaceSlot ps;
+                ps.alive = sidx[{sl.second, ALIVE}];
+                std::map<int, int32_t> adds;
+                adds[ps.alive] += 1;
+                for (int a = 0; a < A; ++a) {
+                    if (rr.created->wrap[a]) adds[sidx[{sl.first, a}]] += (int32_t)rr.created->wrap[a];
+                    if (rr.created->content[a]) adds[sidx[{sl.second, a}]] += (int32_t)rr.created->content[a];
+                }
+                for (auto& kv : adds) ps.adds.push_back({kv.first, kv.second});
+                place.push_back(ps);
+            }
+        fm.place.push_back(place);
+        std::vector<std::pair<int32_t, int32_t>> xf;
+        for (auto& e : rr.xfer) xf.push_back({sidx[e.first], e.second.first >= 0 ? sidx[e.second] : -1});
+        std::sort(xf.begin(), xf.end());
+        fm.transfer.push_back(xf);
     }
-    fm.x_cap_max = max_exact_cap(fm.reactants, (int64_t)1 << 30);
+    // flags are 0/1 and do not limit the exact propensity range (R9)
+    fm.x_cap_max = max_exact_cap(cap_lists, (int64_t)1 << 30);
     return fm;
 }
 

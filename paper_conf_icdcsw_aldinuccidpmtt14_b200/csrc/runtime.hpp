@@ -4,6 +4,7 @@
 #include <cuda.h>
 #include <cuda_runtime.h>
 
+#include <map>
 #include <string>
 #include <vector>
 
@@ -13,6 +14,11 @@
 
 struct cwc_model {
     cwc::FlatModel fm;
+    // load inputs, kept so that "capacity.<label>" can re-flatten (reading R20)
+    std::vector<std::string> in_alphabet, in_rules;
+    std::vector<double> in_rates;
+    std::string in_term;
+    std::map<std::string, int64_t> capacity;
 
     // options (cwc.h)
     int64_t x_cap = 0;
@@ -42,6 +48,8 @@ struct cwc_model {
     // flat-view storage for cwc_model_info
     std::vector<const char*> name_ptrs;
     std::vector<int32_t> info_nreact, info_rspecies, info_rorder, info_delta;
+    std::vector<int32_t> info_place_off, info_place_alive, info_add_off, info_add_s, info_add_n, info_xfer_off,
+        info_xfer_src, info_xfer_dst;
 
     // compiled kernel
     std::string source, nvrtc_log, compiled_key;

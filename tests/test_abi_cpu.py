@@ -52,6 +52,29 @@ def test_compiler_matches_oracle_flattening(name):
     assert info["n_rules"] == len(md.rules)
     assert info["law"] == fm.law and info["law_species"] == fm.law_species
     assert info["law_K"] == fm.law_K and info["law_n"] == fm.law_n
+    # reading R20 (dynamic compartments): gates, placements, transfers, sentinel, flags
+    assert info["gate_species"] == fm.gate_species and info["gate_kind"] == fm.gate_kind
+    assert info["place"] == [[(a, list(ad)) for a, ad in p] for p in fm.place]
+    assert info["transfer"] == [list(t) for t in fm.transfer]
+    assert info["sentinel"] == fm.sentinel and info["flag"] == fm.flag
+
+
+def test_capacity_option_reflattens():
+    """capacity.<label> re-flattens the model (R20) exactly as the oracle does."""
+    m = cwc.Model.from_def(W.VES_TINY)
+    for cap in (1, 5):
+        m.set_option("capacity.v", cap)
+        fm = flatten(W.VES_TINY.species, W.VES_TINY.rules, W.VES_TINY.rates, W.VES_TINY.initial_term,
+                     capacity={"v": cap})
+        info = m.info()
+        assert info["names"] == fm.names and info["delta"] == fm.delta and info["x0"] == fm.x0
+        assert info["place"] == [[(a, list(ad)) for a, ad in p] for p in fm.place]
+    with pytest.raises(cwc.CWCError):
+        m.set_option("capacity.nosuch", 4)      # not a dynamic label
+    with pytest.raises(cwc.CWCError):
+        m.set_option("capacity.v", 0)
+    assert len(m.info()["names"]) == len(flatten(W.VES_TINY.species, W.VES_TINY.rules, W.VES_TINY.rates,
+                                                 W.VES_TINY.initial_term, capacity={"v": 5}).names)
 
 
 REJECT = [
@@ -62,7 +85,10 @@ REJECT = [
     (["top: A -> ."], [float("nan")], "A", 1),
     (["top: A -> ."], [float("inf")], "A", 1),
     (["top: A -> (. $x | $X)^c"], [1.0], "A", 3),
-    (["top: (. $x | $X)^c -> ."], [1.0], "A (.|.)^c", 3),
+    (["top: A -> (.|B)^c (.|B)^c"], [1.0], "A", 3),                # two creations (R20)
+    (["top: A ($x | $X)^c -> A $X ($x | $X)^c"], [1.0], "A", 3),   # release of a kept compartment
+    (["top: A -> (.|B)^c", "c: B -> (.|A)^d"], [1.0, 1.0], "A", 3),  # nested dynamic compartments
+    (["top: ($x | $X)^c -> ."], [1.0], "(. | (.|.)^d)^c", 3),        # dynamic with nested content
     (["top: A A A A -> ."], [1.0], "A", 3),
     (["top: (A | $X)^c -> (. | $X)^c"], [1.0], "A (A|.)^c", 3),
     (["top: (. $x | $X)^c (. $y | $Y)^c -> (. $y | $X)^c (. $x | $Y)^c"], [1.0], "(.|.)^c (.|.)^c", 3),
@@ -141,8 +167,9 @@ def test_nvrtc_compiles_for_sm100a(name):
     src, log = m.compile()
     assert "cwc_ssa_kernel" in src and "__dmul_rn" in src
     attrs = m.kernel_attributes()
-    # spills only around the out-of-line cut emission / slow path are tolerated
-    assert attrs["local_bytes"] <= 512, log
+    # spills only around the out-of-line cut emission / slow path are tolerated; pooled
+    # dynamic-compartment models (R20: ~30 species, ~20 running sums) spill a few in the loop
+    assert attrs["local_bytes"] <= (2048 if W.MODELS[name].capacity else 512), log
     assert 0 < attrs["registers"] <= 255
     # the species state is indexed by compile-time constants only
     body = src[src.index("generated model section"):]

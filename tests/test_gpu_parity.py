@@ -116,6 +116,23 @@ def test_compartments_small():
     _parity(cfg.model, 900, 20.0, cfg.sample_dt, cfg.seed, hist_bins=cfg.hist_bins)
 
 
+def test_vesicles_dynamic_compartments():
+    """SURVEY §8(f)-4 (reading R20): creation into pool slots, dissolution releasing the
+    content, processing inside slots; ragged size, nonzero first."""
+    cfg = W.CONFIGS["vesicles"]
+    _parity(cfg.model, 1500, 40.0, cfg.sample_dt, cfg.seed, first=77_777, hist_bins=cfg.hist_bins)
+
+
+def test_vesicles_pool_overflow_and_quanta():
+    """A 3-slot pool overflows often: full-pool creations freeze instances (OVERFLOWED, R9/R20)
+    identically on both sides, under several quantum sizes."""
+    import dataclasses
+    md = dataclasses.replace(W.VESICLES, capacity=(("ves", 3),))
+    res, *_ = _parity(md, 1200, 60.0, 0.5, 11, hist_bins=256)
+    assert res.overflowed > 50
+    _parity(md, 1200, 60.0, 0.5, 11, hist_bins=256, quantum_samples=5)
+
+
 @pytest.mark.parametrize("name", sorted(W.TINY_MODELS))
 def test_tiny_models(name):
     _parity(W.TINY_MODELS[name], 257, 6.0, 0.25, 99)

@@ -92,7 +92,10 @@ def test_default_cap_keeps_counts_exact():
     (["top: A -> ."], [-1.0], "A", "invalid"),                       # negative rate
     (["top: A -> ."], [float("nan")], "A", "invalid"),
     (["top: A -> (. $x | $X)^c"], [1.0], "A", "unsupported"),        # compartment creation
-    (["top: (. $x | $X)^c -> ."], [1.0], "A (.|.)^c", "unsupported"),  # destruction
+    (["top: A -> (.|B)^c (.|B)^c"], [1.0], "A", "unsupported"),    # two creations in one rule (R20)
+    (["top: A ($x | $X)^c -> A $X ($x | $X)^c"], [1.0], "A", "unsupported"),  # release, not destroyed
+    (["top: A -> (.|B)^c", "c: B -> (.|A)^d"], [1.0, 1.0], "A", "unsupported"),  # nested dynamic
+    (["top: ($x | $X)^c -> ."], [1.0], "(. | (.|.)^d)^c", "unsupported"),  # dynamic with nested compartment
     (["top: A A A A -> ."], [1.0], "A", "unsupported"),              # order > 3
     (["top: (A | $X)^c -> (. | $X)^c"], [1.0], "A (A|.)^c", "unsupported"),  # closed wrap
     (["top: (. $x | $X)^c (. $y | $Y)^c -> (. $y | $X)^c (. $x | $Y)^c"], [1.0],

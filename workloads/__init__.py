@@ -25,6 +25,7 @@ class ModelDef:
     rates: Tuple[float, ...]          # one rate per rule
     initial_term: str
     x_cap: Optional[int] = None       # reading R9; None = model default (largest safe cap <= 2^30)
+    capacity: Tuple[Tuple[str, int], ...] = ()  # reading R20: slots per dynamic-compartment pool
 
 
 @dataclass(frozen=True)
@@ -210,3 +211,42 @@ PERIOD_ANALYSIS = {"neurospora": dict(species="M", lo=100, hi=350, window=48),
 AUTOREPRESSOR = ModelDef("autorepressor", ("P",), ("top: . -> P @ hillr(P, 30, 2)", "top: P -> ."),
                          (60.0, 1.0), ".")
 TINY_MODELS[AUTOREPRESSOR.name] = AUTOREPRESSOR
+
+# --- dynamic compartments (reading R20, bounded pools) ------------------------
+# Vesicle traffic shaped like the paper's compartment creation/destruction: a
+# budding site A creates vesicles loaded with 20 cargo B; cargo is processed to C inside;
+# vesicles fuse with the top level releasing their content; B and C are degraded at the top.
+# Vesicle number is an immigration-death process, Poisson(0.2/0.1 = 2) at stationarity; the
+# pool holds 8 (P(N > 8) ~ 2e-4; a full pool freezes the instance as OVERFLOWED, R9).
+VESICLES = ModelDef(
+    name="vesicles",
+    species=("A", "B", "C"),
+    rules=(
+        "top: A -> A (. | 20*B)^ves",   # budding
+        "ves: B -> C",                  # processing inside a vesicle
+        "top: ($x | $X)^ves -> $X",     # fusion: the content is released to the top level
+        "top: B -> .",
+        "top: C -> .",
+    ),
+    rates=(0.2, 0.2, 0.1, 0.05, 0.05),
+    initial_term="A",
+    capacity=(("ves", 8),),
+)
+MODELS[VESICLES.name] = VESICLES
+CONFIGS["vesicles"] = RunConfig(
+    7, VESICLES, 1_000_000, 100.0, 0.5, SEED_BASE + 7, 1024, 1,
+    description="vesicle traffic with dynamic compartments (R20, 8-slot pool), 1M instances, t_end=100, dt=0.5")
+
+# tiny dynamic models for the term-level CME pin (tests/test_oracle_dynamic.py): creation with
+# cargo, internal decay, dissolution releasing the content, destruction without release
+VES_TINY = ModelDef(
+    "ves_tiny", ("A", "B"),
+    ("top: A -> A (. | B)^v", "v: B -> .", "top: ($x | $X)^v -> $X", "top: B -> ."),
+    (1.0, 0.7, 0.5, 0.3), "A (. | B)^v", capacity=(("v", 3),))
+CELL_KILL = ModelDef(
+    "cell_kill", ("K", "R", "S"),
+    ("top: K -> K (2*R | S)^c", "top: (R $x | $X)^c -> $x", "c: . -> S", "top: (. $x | S $X)^c -> .",
+     "top: R -> ."),
+    (0.8, 0.4, 0.6, 0.3, 0.5), "K (2*R | S)^c", capacity=(("c", 2),))
+TINY_MODELS[VES_TINY.name] = VES_TINY
+TINY_MODELS[CELL_KILL.name] = CELL_KILL
