@@ -92,6 +92,15 @@ def test_lv_short_horizon_ragged():
     _parity(cfg.model, 1537, 2.0, cfg.sample_dt, cfg.seed, hist_bins=cfg.hist_bins, hist_width=cfg.hist_width)
 
 
+def test_terminated_instances_under_quanta():
+    """Absorbed / overflowed instances end in an early quantum; every later quantum item of the
+    instance must be skipped (regression: the third quantum waited forever)."""
+    cfg = W.CONFIGS["lv"]
+    res, *_ = _parity(cfg.model, 400, 50.0, 0.5, cfg.seed + 7, hist_bins=cfg.hist_bins, hist_width=cfg.hist_width,
+                      quantum_samples=4)
+    assert res.overflowed > 0 and res.absorbed > 0
+
+
 def test_lv_long_horizon_absorb_and_overflow():
     # long horizon: predator extinction, prey runaway past X_cap (R9) and full extinction (R8)
     cfg = W.CONFIGS["lv"]
