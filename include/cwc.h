@@ -146,7 +146,7 @@ cwc_status cwc_model_info(cwc_model_t m, cwc_model_info_t* out);
  *                        Re-flattens the model: set it first (species-indexed options such as
  *                        hist_width.<name>, period_species and x_cap are reset).   default 8
  *   "x_cap"              1 <= v <= x_cap_max (R9).                       default x_cap_max or model's
- *   "raw_samples"        0/1: keep the raw [T][S][count] int32 sample buffer.   default 1
+ *   "raw_samples"        0/1: keep the raw int32 sample buffer (cwc_samples).       default 1
  *   "hist_bins"          B >= 1 in-range bins per (time, species).               default 256
  *   "hist_width"         bin width >= 1 for every species;  "hist_width.<species name>" for one.
  *   "hist_lo"            left edge of bin 1 for every species; "hist_lo.<species name>" for one.
@@ -183,7 +183,9 @@ cwc_status cwc_kernel_attributes(cwc_model_t m, int32_t* regs, int32_t* local_by
  * Device buffers.  By default the handle allocates what it needs.  A caller that owns device
  * memory (PyTorch) may bind its own buffers instead; they must stay valid while bound.
  *   stats   int64[stats_len]   packed ensemble statistics (layout below)
- *   raw     int32[raw_len]     raw samples [T][S][count] (only if raw_samples = 1)
+ *   raw     int32[raw_len]     raw samples (only if raw_samples = 1), time-blocked SoA
+ *                              [ceil(T/8)][S][count][8]: cut k of species s of local instance i
+ *                              at ((k/8*S + s)*count + i)*8 + k%8 (cwc_samples returns [T][S][count])
  *   scratch bytes              per-instance state + work queue
  * cwc_buffer_sizes reports the sizes one cwc_simulate_range(count, t_end, dt) needs.
  * Passing NULL pointers to cwc_bind_device_buffers unbinds (back to library allocation).

@@ -23,7 +23,7 @@ struct cwc_params {
     int pad0;
     cwc_round_keys rk;          // Philox round keys of the seed
     unsigned long long* stats;  // packed int64 stats (cwc.h layout)
-    int* raw;                   // [T][S][count] or nullptr
+    int* raw;                   // [ceil(T/8)][S][count][8] (time-blocked SoA) or nullptr
     int* st_x;                  // [S][count] saved species counts
     double* st_t;               // [count] saved time
     unsigned long long* st_step;  // [count] saved step (= reactions applied)
@@ -39,3 +39,6 @@ struct cwc_params {
 };
 
 #define CWC_TERMINAL 0x80000000u
+// raw cuts per 32-byte block of one (species, instance): a lane fills the whole sector while it
+// is resident in L2, so the sample stream reaches DRAM as full sectors (no read-for-fill)
+#define CWC_RAW_BLOCK 8

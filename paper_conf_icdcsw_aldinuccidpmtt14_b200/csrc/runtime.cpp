@@ -119,7 +119,7 @@ static ScratchLayout scratch_layout(int S, int64_t count, int64_t T) {
 void buffer_sizes(const cwc_model* m, int64_t count, int64_t K, size_t* stats, size_t* raw, size_t* scratch) {
     const int S = m->fm.S();
     if (stats) *stats = stats_len(K + 1, S, m->hist_bins, m->period_species >= 0);
-    if (raw) *raw = m->raw_samples ? (size_t)(K + 1) * S * (size_t)count : 0;
+    if (raw) *raw = m->raw_samples ? (size_t)((K + CWC_RAW_BLOCK) / CWC_RAW_BLOCK) * CWC_RAW_BLOCK * S * (size_t)count : 0;
     if (scratch) *scratch = scratch_layout(S, count, K + 1).total;
 }
 
@@ -641,10 +641,19 @@ void copy_samples(cwc_model* m, int64_t first, int64_t count, int32_t* out) {
     if (!out) fail(CWC_E_INVALID, "null output");
     ck(cudaStreamSynchronize(m->last_stream), "simulation");
     if (count == 0) return;
-    const size_t rows = (size_t)(m->K + 1) * m->fm.S();
-    ck(cudaMemcpy2D(out, (size_t)count * 4, m->d_raw + first, (size_t)m->count * 4, (size_t)count * 4, rows,
-                    cudaMemcpyDeviceToHost),
+    // device layout [ceil(T/8)][S][m->count][8] (time-blocked) -> out[T][S][count]
+    const int64_t S = m->fm.S(), T = m->K + 1, TB = (T + CWC_RAW_BLOCK - 1) / CWC_RAW_BLOCK;
+    const size_t row = (size_t)count * CWC_RAW_BLOCK;
+    std::vector<int32_t> tmp((size_t)TB * S * row);
+    ck(cudaMemcpy2D(tmp.data(), row * 4, m->d_raw + first * CWC_RAW_BLOCK, (size_t)m->count * CWC_RAW_BLOCK * 4,
+                    row * 4, (size_t)TB * S, cudaMemcpyDeviceToHost),
        "copy samples");
+    for (int64_t k = 0; k < T; ++k)
+        for (int64_t s = 0; s < S; ++s) {
+            const int32_t* src = tmp.data() + ((size_t)(k / CWC_RAW_BLOCK) * S + s) * row + (k % CWC_RAW_BLOCK);
+            int32_t* dst = out + ((size_t)k * S + s) * count;
+            for (int64_t j = 0; j < count; ++j) dst[j] = src[(size_t)j * CWC_RAW_BLOCK];
+        }
 }
 
 void copy_records(cwc_model* m, int64_t first, int64_t count, uint8_t* flags, int64_t* reactions, double* t_last) {

@@ -155,7 +155,7 @@ def test_buffer_sizes_layout():
     n_stats, n_raw, n_scratch = m.buffer_sizes(1000, 50.0, 0.1)
     T, S, B = 501, 2, 1024
     assert n_stats == T * (1 + 3 * S + S * (B + 2)) + _lib.N_CTR
-    assert n_raw == T * S * 1000
+    assert n_raw == -(-T // 8) * 8 * S * 1000   # time-blocked [ceil(T/8)][S][count][8]
     assert n_scratch >= 1000 * (S * 4 + 8 + 8 + 8 + 4 + 4)
     m.set_option("raw_samples", 0)
     assert m.buffer_sizes(1000, 50.0, 0.1)[1] == 0
