@@ -178,6 +178,10 @@ cwc_status cwc_model_compile(cwc_model_t m, const char** source, const char** lo
 /* Compiled SASS-level facts of the last compile: registers/thread, local (spill) bytes. */
 cwc_status cwc_kernel_attributes(cwc_model_t m, int32_t* regs, int32_t* local_bytes,
                                  int32_t* max_threads);
+/* The compiled sm_100a kernel image (cubin) the module is loaded from: a borrowed view, valid
+ * until the next compile or cwc_model_free; either pointer may be NULL.  CWC_E_STATE before the
+ * first compile. */
+cwc_status cwc_kernel_image(cwc_model_t m, const void** image, size_t* bytes);
 
 /* ------------------------------------------------------------------------------------------
  * Device buffers.  By default the handle allocates what it needs.  A caller that owns device

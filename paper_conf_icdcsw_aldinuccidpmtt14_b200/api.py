@@ -186,6 +186,12 @@ class Model:
         check(lib.cwc_kernel_attributes(self._h, ctypes.byref(r), ctypes.byref(l), ctypes.byref(t)))
         return dict(registers=r.value, local_bytes=l.value, max_threads=t.value)
 
+    def kernel_image_bytes(self) -> int:
+        """Size of the compiled sm_100a cubin (uploaded to the device at module load)."""
+        n = ctypes.c_size_t()
+        check(lib.cwc_kernel_image(self._h, None, ctypes.byref(n)))
+        return n.value
+
     def buffer_sizes(self, count: int, t_end: float, dt: float):
         a, b, c = ctypes.c_size_t(), ctypes.c_size_t(), ctypes.c_size_t()
         check(lib.cwc_buffer_sizes(self._h, int(count), float(t_end), float(dt), ctypes.byref(a), ctypes.byref(b),

@@ -309,6 +309,15 @@ cwc_status cwc_kernel_attributes(cwc_model_t m, int32_t* regs, int32_t* local_by
     });
 }
 
+cwc_status cwc_kernel_image(cwc_model_t m, const void** image, size_t* bytes) {
+    return guard([&] {
+        need(m != nullptr, "NULL model");
+        if (m->cubin.empty()) fail(CWC_E_STATE, "kernel not compiled");
+        if (image) *image = m->cubin.data();
+        if (bytes) *bytes = m->cubin.size();
+    });
+}
+
 cwc_status cwc_buffer_sizes(cwc_model_t m, int64_t count, double t_end, double dt, size_t* stats, size_t* raw,
                             size_t* scratch) {
     return guard([&] {

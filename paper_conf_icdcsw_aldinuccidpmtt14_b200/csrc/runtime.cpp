@@ -16,6 +16,10 @@
 #include <fstream>
 #include <mutex>
 #include <dlfcn.h>
+
+// bench.py counts the launch parameter block in its end-to-end H2D bytes (PARAM_BYTES)
+static_assert(sizeof(cwc_params) == 240, "cwc_params layout changed: update bench.py PARAM_BYTES");
+static_assert(sizeof(cwc_logtab_entry) * 128 == 3072, "log table size");
 #include <sstream>
 #include <sys/stat.h>
 #include <unistd.h>

@@ -171,6 +171,12 @@ def test_nvrtc_compiles_for_sm100a(name):
     # dynamic-compartment models (R20: ~30 species, ~20 running sums) spill a few in the loop
     assert attrs["local_bytes"] <= (2048 if W.MODELS[name].capacity else 512), log
     assert 0 < attrs["registers"] <= 255
+    # the image is an sm_100a ELF cubin (what the module upload sends to the device)
+    import ctypes
+    from paper_conf_icdcsw_aldinuccidpmtt14_b200 import _lib
+    img, n = ctypes.c_void_p(), ctypes.c_size_t()
+    assert _lib.lib.cwc_kernel_image(m._h, ctypes.byref(img), ctypes.byref(n)) == 0
+    assert n.value == m.kernel_image_bytes() > 1024 and ctypes.string_at(img, 4) == b"\x7fELF"
     # the species state is indexed by compile-time constants only
     body = src[src.index("generated model section"):]
     assert "x[j]" not in body and "x[s]" not in body.split("cwc_bin")[0]
