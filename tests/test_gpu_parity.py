@@ -187,20 +187,24 @@ def test_sharding_invariance():
 
 
 # ------------------------------------------------------------------ bench-size runs, sampled
-@pytest.mark.parametrize("cname", ["lv", "schlogl"])
-def test_full_size_sampled(cname):
+@pytest.mark.parametrize("cname,shards", [("lv", 1), ("schlogl", 1), ("compartments", 1), ("circadian", 8)])
+def test_full_size_sampled(cname, shards):
+    """BASELINE sizes in the bench's launch configuration; circadian (10M over 8 GPUs) as the last
+    1.25M shard, so instance ids (the Philox key) are global ones far from 0."""
     cfg = W.CONFIGS[cname]
     N = cfg.n_instances
-    res, raw, flags, reactions, m = gpu_run(cfg.model, N, 0, N, cfg.t_end, cfg.sample_dt, cfg.seed,
+    first = (shards - 1) * N // shards
+    count = N - first
+    res, raw, flags, reactions, m = gpu_run(cfg.model, N, first, count, cfg.t_end, cfg.sample_dt, cfg.seed,
                                             hist_bins=cfg.hist_bins, hist_width=cfg.hist_width, quantiles=QS)
-    assert res.finished == N
+    assert res.finished == count
     assert_stats_match_raw(res, raw)
     rng = np.random.default_rng(0)
-    pick = sorted(set([0, 1, N - 1] + list(rng.integers(0, N, 29))))
+    pick = sorted(set([0, 1, count - 1] + list(rng.integers(0, count, 29))))
     fm = flatten_def(cfg.model)
     cm = oracle.CModel(fm)
     for i in pick:
-        o = oracle.simulate(cm, i, 1, cfg.t_end, cfg.sample_dt, cfg.seed)
+        o = oracle.simulate(cm, first + i, 1, cfg.t_end, cfg.sample_dt, cfg.seed)
         assert np.array_equal(raw[:, :, i], o.raw[:, :, 0]), i
         assert reactions[i] == o.reactions[0] and flags[i] == o.flags[0]
     assert res.reactions == int(reactions.sum())
