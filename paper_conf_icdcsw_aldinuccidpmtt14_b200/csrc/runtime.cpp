@@ -16,10 +16,21 @@
 #include <fstream>
 #include <mutex>
 #include <dlfcn.h>
+#include <nvtx3/nvToolsExt.h>  // header-only NVTX v3: ranges are free unless a profiler injects
 
 // bench.py counts the launch parameter block in its end-to-end H2D bytes (PARAM_BYTES)
 static_assert(sizeof(cwc_params) == 240, "cwc_params layout changed: update bench.py PARAM_BYTES");
 static_assert(sizeof(cwc_logtab_entry) * 128 == 3072, "log table size");
+
+namespace {
+// NVTX range over a host-side phase of the path (visible in nsys / ncu --nvtx timelines)
+struct NvtxRange {
+    explicit NvtxRange(const char* name) { nvtxRangePushA(name); }
+    ~NvtxRange() { nvtxRangePop(); }
+    NvtxRange(const NvtxRange&) = delete;
+    NvtxRange& operator=(const NvtxRange&) = delete;
+};
+}  // namespace
 #include <sstream>
 #include <sys/stat.h>
 #include <unistd.h>
@@ -220,6 +231,7 @@ static void parse_ptxas(cwc_model* m) {
 }
 
 void compile(cwc_model* m, const uint64_t* seed) {
+    NvtxRange nvtx_range("cwc_model_compile");
     KernelConfig cfg;
     cfg.block_threads = m->block_threads;
     // auto register budget: 768 resident threads per SM (<= 80 registers) — measured best for the
@@ -383,6 +395,7 @@ static void grow(T*& p, size_t& cap, size_t need_bytes, const char* what) {
 
 void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count, double t_end, double dt,
                     uint64_t seed, cudaStream_t stream, bool own_stream) {
+    NvtxRange nvtx_range("cwc_simulate_range");
     if (n_total <= 0) fail(CWC_E_INVALID, "n_total must be > 0");
     if (first < 0 || count < 0 || first + count > n_total) fail(CWC_E_INVALID, "instance range outside [0, n_total)");
     const int64_t K = grid_K(t_end, dt);
@@ -534,6 +547,7 @@ static double quantile_from_hist(const int64_t* h, int B, int64_t n, double q, i
 static void derive(cwc_model* m);
 
 void finalize(cwc_model* m, const int64_t* host_stats) {
+    NvtxRange nvtx_range("cwc_stats_finalize");
     if (!m->simulated) fail(CWC_E_STATE, "no simulation to finalize");
     const size_t len = m->last_stats_len;
     m->h_stats.resize(len);
@@ -552,6 +566,7 @@ void finalize(cwc_model* m, const int64_t* host_stats) {
 // (an instance that ended early emitted or filled all its later cuts).  The counters are read
 // before the statistics, so the snapshot contains every update of the cuts it reports final.
 void snapshot(cwc_model* m, int64_t* cuts_final, int64_t* items_done) {
+    NvtxRange nvtx_range("cwc_stats_snapshot");
     if (!m->simulated) fail(CWC_E_STATE, "no simulation");
     if (!m->stream) fail(CWC_E_STATE, "snapshots need the \"stream\" option set before simulating");
     if (!m->poll_stream) ck(cudaStreamCreateWithFlags(&m->poll_stream, cudaStreamNonBlocking), "cudaStreamCreate");
@@ -639,6 +654,7 @@ static void derive(cwc_model* m) {
 }
 
 void copy_samples(cwc_model* m, int64_t first, int64_t count, int32_t* out) {
+    NvtxRange nvtx_range("cwc_samples");
     if (!m->simulated) fail(CWC_E_STATE, "no simulation");
     if (!m->raw_samples || !m->d_raw) fail(CWC_E_STATE, "raw samples are disabled");
     if (first < 0 || count < 0 || first + count > m->count) fail(CWC_E_INVALID, "range outside the last simulation");
