@@ -147,6 +147,24 @@ def test_tiny_models(name):
     _parity(W.TINY_MODELS[name], 257, 6.0, 0.25, 99)
 
 
+def test_empty_shard():
+    """A rank whose contiguous share is empty (n_total < world): a valid no-op whose statistics
+    are all zero and sum neutrally into the all-reduce."""
+    import paper_conf_icdcsw_aldinuccidpmtt14_b200 as cwc
+    m = cwc.Model.from_def(W.LOTKA_VOLTERRA, hist_bins=64)
+    m.simulate_range(3, 3, 0, 1.0, 0.1, 9)
+    res = m.finalize()
+    assert res.finished == 0 and res.reactions == 0
+    assert not res.n.any() and not res.sum.any() and not res.hist.any()
+    assert np.isnan(res.mean).all()
+
+
+def test_many_cuts_global_moments():
+    """T = 20,001 cuts: the moment accumulators no longer fit in shared memory, so the kernel
+    records straight into the global buffer (the other recording path)."""
+    _parity(W.IMM_DEATH, 300, 2000.0, 0.1, 77, hist_bins=300)
+
+
 def test_zero_horizon_and_single_instance():
     _parity(W.LOTKA_VOLTERRA, 1, 0.0, 0.1, 5)
     _parity(W.SCHLOGL, 1, 3.0, 0.1, 5)
