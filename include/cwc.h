@@ -160,6 +160,10 @@ cwc_status cwc_model_info(cwc_model_t m, cwc_model_info_t* out);
  *   "stream"             0/1: on-line streaming — progress counters + cwc_stats_snapshot.
  *   "smem_stats"         0/1: accumulate n/sum/sumsq per CTA in shared memory and flush once
  *                        (used when T*(1+3S)*8 bytes fit without lowering residency). default 1
+ *   "fast_cut"           -1/0/1: where cuts are recorded — inside the fast step (1) or on the
+ *                        full-step path (0); -1 = auto: 0 when the last simulation on this handle
+ *                        (else a0(x0)*sample_dt) had >= 1000 reactions per recorded cut.
+ *                        Performance only: results are bit-identical.             default -1
  *   "seed_jit"           0/1: specialise the kernel on the seed (Philox round keys become
  *                        instruction immediates; one NVRTC compile per new seed, cached).
  *   "refill"             0/1: warp-level refill from the global work queue.      default 1

@@ -260,6 +260,9 @@ cwc_status cwc_set_option_i64(cwc_model_t m, const char* key, int64_t v) {
         } else if (k == "ilp") {
             need(v == 1 || v == 2, "ilp is 1 or 2");
             m->ilp = (int)v;
+        } else if (k == "fast_cut") {
+            need(v >= -1 && v <= 1, "fast_cut is -1 (auto), 0 or 1");
+            m->fast_cut = (int)v;
         } else if (k == "seed_jit") {
             need(v == 0 || v == 1, "seed_jit is 0 or 1");
             m->seed_jit = (int)v;

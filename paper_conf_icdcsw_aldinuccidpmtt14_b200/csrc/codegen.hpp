@@ -19,6 +19,7 @@ struct KernelConfig {
     int period_species = -1;  // on-line period detector on this flat species (-1 = off)
     int64_t period_lo = 0, period_hi = 1;
     int64_t x_cap = 0;
+    bool fast_cut = true;  // the fast step records a due cut itself (else it leaves the fast loop)
     std::vector<int64_t> hist_lo, hist_width;  // [S]
 };
 

@@ -244,6 +244,7 @@ void compile(cwc_model* m, const uint64_t* seed) {
     cfg.period_hi = m->period_hi;
     cfg.hist_bins = m->hist_bins;
     cfg.x_cap = m->x_cap;
+    cfg.fast_cut = m->fast_cut_now;
     cfg.hist_lo = m->hist_lo;
     cfg.hist_width = m->hist_width;
     if (seed && m->seed_jit) {
@@ -393,6 +394,42 @@ static void grow(T*& p, size_t& cap, size_t need_bytes, const char* what) {
     cap = need_bytes;
 }
 
+// Expected reactions between two cuts from the initial state: a0(x0) * dt (functional laws
+// evaluated at x0, gates ignored) — only the first guess of choose_fast_cut.
+static double a0_estimate(const FlatModel& fm) {
+    double a0 = 0;
+    for (int j = 0; j < fm.M(); ++j) {
+        double h = 1;
+        for (const Reactant& r : fm.reactants[j]) {
+            const double x = fm.x0[r.species];
+            for (int i = 0; i < r.order; ++i) h *= (x - i) / (i + 1);
+            if (h <= 0) { h = 0; break; }
+        }
+        double a = fm.rates[j] * h;
+        if (!fm.law.empty() && fm.law[j] != 0 && fm.law_species[j] >= 0) {
+            const double X = fm.x0[fm.law_species[j]], K = fm.law_K[j], n = fm.law.size() ? fm.law_n[j] : 1;
+            const double Xn = std::pow(X, n), Kn = std::pow(K, n);
+            if (fm.law[j] == 1) a = h > 0 ? fm.rates[j] * X / (K + X) : 0;
+            else if (fm.law[j] == 2) a = h > 0 ? fm.rates[j] * Xn / (Kn + Xn) : 0;
+            else a = h > 0 ? fm.rates[j] * Kn / (Kn + Xn) : 0;
+        }
+        a0 += a;
+    }
+    return a0;
+}
+
+// Where the fast step records cuts.  Inline (1) costs the fast loop a call site, which makes
+// ptxas rematerialise constants and shuffle registers every step; leaving the fast loop for the
+// full step (0) costs a warp-wide exit per recorded cut.  Same-box A/B (profiles/
+// r1h_ab_fast_cut.log): leaving wins from ~1,000 reactions per cut (LV 2,800: -2.9 %, circadian
+// 1,400: -2.0 %) and loses below (Schlogl 490: +1.2 %, Neurospora 610: +7.6 %, compartments
+// 290: +6.3 %).  Auto decides by the last run on this handle, else by a0(x0) * dt.
+static bool choose_fast_cut(cwc_model* m, double dt) {
+    if (m->fast_cut >= 0) return m->fast_cut != 0;
+    const double rpc = m->last_reactions_per_cut > 0 ? m->last_reactions_per_cut : a0_estimate(m->fm) * dt;
+    return rpc < 1000.0;
+}
+
 void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count, double t_end, double dt,
                     uint64_t seed, cudaStream_t stream, bool own_stream) {
     NvtxRange nvtx_range("cwc_simulate_range");
@@ -403,6 +440,7 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
         fail(CWC_E_INVALID, "period analysis needs period_lo < period_hi");
     const int64_t T = K + 1;
     const int S = m->fm.S();
+    m->fast_cut_now = choose_fast_cut(m, dt);
     compile(m, &seed);
     const int dev = current_device(m);
     ensure_module(m, dev);
@@ -558,6 +596,13 @@ void finalize(cwc_model* m, const int64_t* host_stats) {
     else ck(cudaMemcpy(m->h_stats.data(), m->d_stats, len * 8, cudaMemcpyDeviceToHost), "copy stats");
     m->cuts_final = m->K + 1;
     derive(m);
+    {   // reactions per recorded cut of this run (choose_fast_cut of the next simulation)
+        int64_t recs = 0;
+        for (int64_t v : m->h_n) recs += v;
+        const int64_t T = m->K + 1, TS = T * m->fm.S(), B = m->hist_bins;
+        const int64_t reactions = m->h_stats[T + 3 * TS + TS * (B + 2) + CWC_CTR_REACTIONS];
+        if (recs > 0) m->last_reactions_per_cut = (double)reactions / (double)recs;
+    }
 }
 
 // On-line streaming: while the kernel

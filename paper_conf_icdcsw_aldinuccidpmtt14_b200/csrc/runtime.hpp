@@ -32,6 +32,11 @@ struct cwc_model {
     int ilp = 1;
     int delta_table = -1;
     int smem_stats = 1;
+    // cut recording inside the fast step (1) or on the full-step path (0); -1 = auto: by the
+    // reactions per recorded cut of the last simulation on this handle (else a0(x0) * dt)
+    int fast_cut = -1;
+    double last_reactions_per_cut = 0;
+    bool fast_cut_now = true;             // the mode of the kernel being compiled / launched
     // on-line period analysis (reading R19): observable species (-1 = off), Schmitt thresholds,
     // moving-average window in cuts
     int period_species = -1;

@@ -87,9 +87,12 @@ def test_config1_imm_death_full():
             hist_width=cfg.hist_width)
 
 
-def test_lv_short_horizon_ragged():
+@pytest.mark.parametrize("fast_cut", [-1, 0, 1])
+def test_lv_short_horizon_ragged(fast_cut):
+    # LV has ~3,000 reactions per cut: auto (-1) records cuts on the full-step path (0)
     cfg = W.CONFIGS["lv"]
-    _parity(cfg.model, 1537, 2.0, cfg.sample_dt, cfg.seed, hist_bins=cfg.hist_bins, hist_width=cfg.hist_width)
+    _parity(cfg.model, 1537, 2.0, cfg.sample_dt, cfg.seed, hist_bins=cfg.hist_bins, hist_width=cfg.hist_width,
+            fast_cut=fast_cut)
 
 
 def test_terminated_instances_under_quanta():
@@ -175,6 +178,7 @@ def test_schedule_invariance():
     md = W.SCHLOGL
     base = None
     for opts in ({}, {"quantum_samples": 1}, {"quantum_samples": 7}, {"block_threads": 128},
+                 {"fast_cut": 0}, {"fast_cut": 1, "quantum_samples": 3},
                  {"block_threads": 512, "quantum_samples": 2}, {"refill": False}, {"blocks_per_sm": 1}):
         res, raw, flags, reactions, _ = gpu_run(md, 5000, 0, 5000, 4.0, 0.1, 42, hist_bins=512, **opts)
         cur = (res.n, res.sum, res.sqlo, res.sqhi, res.hist, raw, reactions)
