@@ -244,7 +244,7 @@ void compile(cwc_model* m, const uint64_t* seed) {
     cfg.period_hi = m->period_hi;
     cfg.hist_bins = m->hist_bins;
     cfg.x_cap = m->x_cap;
-    cfg.fast_cut = m->fast_cut_now;
+    cfg.fast_cut = m->fast_cut >= 0 ? m->fast_cut != 0 : m->fast_cut_now;  // explicit option wins
     cfg.hist_lo = m->hist_lo;
     cfg.hist_width = m->hist_width;
     if (seed && m->seed_jit) {
