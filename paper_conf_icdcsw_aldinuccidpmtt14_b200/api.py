@@ -73,6 +73,7 @@ class Model:
         check(lib.cwc_model_load(ctypes.byref(h), len(species), sp, len(rules), rl, rt, initial_term.encode()))
         self._h = h
         self._info_cache = None
+        self._bound_buffers = None   # DeviceBuffers bound to the handle (kept alive while bound)
         for label, c in dict(capacity or {}).items():   # re-flattens: before species options (R20)
             self.set_option(f"capacity.{label}", int(c))
         if x_cap is not None:
@@ -121,6 +122,7 @@ class Model:
         if getattr(self, "_h", None):
             lib.cwc_model_free(self._h)
             self._h = None
+        self._bound_buffers = None
 
     def __del__(self):
         try:
@@ -326,9 +328,15 @@ class DeviceBuffers:
             model.handle, ctypes.c_void_p(self.stats.data_ptr()), n_stats,
             ctypes.c_void_p(self.raw.data_ptr() if self.raw is not None else 0), n_raw,
             ctypes.c_void_p(self.scratch.data_ptr()), n_scratch))
+        # the library keeps raw pointers into these tensors: the model holds the buffers alive
+        # while they are bound (results, samples and records read them after the caller's
+        # DeviceBuffers / ShardedRun object is gone)
+        model._bound_buffers = self
 
     def unbind(self):
         check(lib.cwc_bind_device_buffers(self.model.handle, None, 0, None, 0, None, 0))
+        if getattr(self.model, "_bound_buffers", None) is self:
+            self.model._bound_buffers = None
 
 
 def selftest_philox(ctr: np.ndarray, key: np.ndarray) -> np.ndarray:

@@ -150,6 +150,23 @@ def test_tiny_models(name):
     _parity(W.TINY_MODELS[name], 257, 6.0, 0.25, 99)
 
 
+def test_results_outlive_sharded_run():
+    """dist.simulate_sharded binds torch-owned buffers; samples read after its run object is
+    gone (and after torch reuses freed memory) must still be the simulation's."""
+    import gc
+    import torch
+    import paper_conf_icdcsw_aldinuccidpmtt14_b200 as cwc
+    from paper_conf_icdcsw_aldinuccidpmtt14_b200 import dist as cdist
+    m = cwc.Model.from_def(W.IMM_DEATH, hist_bins=256)
+    cdist.simulate_sharded(m, 500, 100.0, 1.0, 3)
+    gc.collect()
+    junk = torch.full((64 << 20,), -7, dtype=torch.int32, device="cuda")
+    torch.cuda.synchronize()
+    raw = m.samples(0, 500)
+    del junk
+    assert np.array_equal(raw, _oracle(W.IMM_DEATH, 0, 500, 100.0, 1.0, 3).raw)
+
+
 def test_empty_shard():
     """A rank whose contiguous share is empty (n_total < world): a valid no-op whose statistics
     are all zero and sum neutrally into the all-reduce."""
