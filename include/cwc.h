@@ -260,6 +260,24 @@ cwc_status cwc_stats_finalize(cwc_model_t m, const int64_t* host_stats);
  * work items.  Moments then accumulate in global memory (no CTA-local staging).
  * Errors: CWC_E_STATE without a simulation or without "stream". */
 cwc_status cwc_stats_snapshot(cwc_model_t m, int64_t* cuts_final, int64_t* items_done);
+/* Terminate the running simulation (Fig. 2, "start new simulations, steer and
+ * terminate running simulations"; "stream" option only).  The kernel stops handing out work
+ * items; items in flight finish their quantum.  Returns without waiting; cwc_stats_finalize then
+ * waits for the kernel and reports in cuts_final the prefix of cuts every instance reached (those
+ * statistics are exact; later cuts are partial).  Errors: CWC_E_STATE without a streaming
+ * simulation. */
+cwc_status cwc_cancel(cwc_model_t m);
+/* The packed statistics (layout above) behind the current cwc_stats views, as copied by the last
+ * snapshot or finalize: a borrowed host view valid until the next snapshot / finalize / load /
+ * simulate / free.  CWC_E_STATE before the first snapshot or finalize. */
+cwc_status cwc_stats_host(cwc_model_t m, const int64_t** host_stats, size_t* n_int64);
+/* Replace the host statistics by a packed buffer of the last simulation's geometry (copied) and
+ * re-derive the cwc_stats views with cuts [0, cuts_final) marked final — the multi-GPU on-line
+ * path: every rank snapshots its running shard, the packed buffers are summed and the final-cut
+ * prefixes min-reduced across ranks (dist.snapshot_sharded), and each rank loads the combined
+ * partial result.  No device synchronisation.  Errors: CWC_E_STATE without a simulation;
+ * CWC_E_INVALID for a null buffer or cuts_final outside [0, T]. */
+cwc_status cwc_stats_load(cwc_model_t m, const int64_t* host_stats, int64_t cuts_final);
 
 typedef struct {
     int32_t T, S, B, n_q;

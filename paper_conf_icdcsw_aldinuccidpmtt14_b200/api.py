@@ -254,10 +254,28 @@ class Model:
         check(lib.cwc_stats_snapshot(self._h, ctypes.byref(cf), ctypes.byref(done)))
         return cf.value, done.value, self.stats()
 
+    def stats_host(self) -> np.ndarray:
+        """Copy of the packed statistics behind the current views (last snapshot / finalize)."""
+        p, n = ctypes.c_void_p(), ctypes.c_size_t()
+        check(lib.cwc_stats_host(self._h, ctypes.byref(p), ctypes.byref(n)))
+        return np.ctypeslib.as_array(ctypes.cast(p, ctypes.POINTER(ctypes.c_int64)), shape=(n.value,)).copy()
+
+    def stats_load(self, packed: np.ndarray, cuts_final: int) -> "EnsembleResult":
+        """Load a packed statistics buffer (e.g. summed over ranks) as the current result."""
+        buf = np.ascontiguousarray(packed, dtype=np.int64)
+        check(lib.cwc_stats_load(self._h, _ptr(buf), int(cuts_final)))
+        return self.stats()
+
+    def cancel(self):
+        """Terminate the running streaming simulation (cwc_cancel)."""
+        check(lib.cwc_cancel(self._h))
+
     def stream(self, n_instances: int, t_end: float, sample_dt: float, seed: int, poll_s: float = 0.02,
-               stream=None):
+               stream=None, stop=None):
         """On-line streaming: launch, then yield (cuts_final, partial result) each
-        time more cuts become final, and finally (T, finalised result)."""
+        time more cuts become final, and finally (cuts_final, finalised result) — cuts_final = T
+        unless ``stop(cuts_final, partial_result)`` returned True, which terminates the running
+        simulation (steering) and finalises the cuts completed so far."""
         import time
         self.set_option("stream", 1)
         self.simulate_range(n_instances, 0, n_instances, t_end, sample_dt, seed, stream=stream)
@@ -269,10 +287,14 @@ class Model:
                 last = cf
                 if cf < T:
                     yield cf, res
+                    if stop is not None and stop(cf, res):
+                        self.cancel()
+                        break
             if cf >= T:
                 break
             time.sleep(poll_s)
-        yield T, self.finalize()
+        res = self.finalize()
+        yield res.cuts_final, res
 
     def period_stats(self) -> dict:
         """On-line period analysis of the last simulation (cwc_period_stats) as numpy arrays."""

@@ -370,6 +370,29 @@ cwc_status cwc_stats_snapshot(cwc_model_t m, int64_t* cuts_final, int64_t* items
     });
 }
 
+cwc_status cwc_stats_host(cwc_model_t m, const int64_t** host_stats, size_t* n_int64) {
+    return guard([&] {
+        need(m != nullptr, "NULL model");
+        if (m->h_stats.empty()) fail(CWC_E_STATE, "no snapshot / finalize yet");
+        if (host_stats) *host_stats = m->h_stats.data();
+        if (n_int64) *n_int64 = m->h_stats.size();
+    });
+}
+
+cwc_status cwc_stats_load(cwc_model_t m, const int64_t* host_stats, int64_t cuts_final) {
+    return guard([&] {
+        need(m != nullptr, "NULL model");
+        cwc::load_host_stats(m, host_stats, cuts_final);
+    });
+}
+
+cwc_status cwc_cancel(cwc_model_t m) {
+    return guard([&] {
+        need(m != nullptr, "NULL model");
+        cwc::cancel(m);
+    });
+}
+
 cwc_status cwc_stats_finalize(cwc_model_t m, const int64_t* host_stats) {
     return guard([&] {
         need(m != nullptr, "NULL model");

@@ -33,6 +33,7 @@ struct cwc_params {
     unsigned int* st_qdone;     // [count] quanta completed (release/acquire)
     unsigned long long* work;   // work-queue counter
     unsigned int* qprog;        // [n_quanta] finished items per quantum (streaming progress) or null
+    const unsigned int* cancel; // streaming only: set by the host (cwc_cancel) to stop taking items
     const cwc_logtab_entry* logtab;  // [128]
     long long smem_stats;       // 1: n/sum/sumsq accumulate per CTA in dynamic shared memory
                                 //    (T*(1+3S) u64) and are flushed once at the end

@@ -19,7 +19,7 @@
 #include <nvtx3/nvToolsExt.h>  // header-only NVTX v3: ranges are free unless a profiler injects
 
 // bench.py counts the launch parameter block in its end-to-end H2D bytes (PARAM_BYTES)
-static_assert(sizeof(cwc_params) == 240, "cwc_params layout changed: update bench.py PARAM_BYTES");
+static_assert(sizeof(cwc_params) == 248, "cwc_params layout changed: update bench.py PARAM_BYTES");
 static_assert(sizeof(cwc_logtab_entry) * 128 == 3072, "log table size");
 
 namespace {
@@ -111,7 +111,7 @@ size_t stats_len(int64_t T, int S, int B, bool period) {
 static size_t align256(size_t v) { return (v + 255) & ~(size_t)255; }
 
 struct ScratchLayout {
-    size_t x, t, step, k, flags, pd, qdone, work, qprog, total;
+    size_t x, t, step, k, flags, pd, qdone, work, cancel, qprog, total;
 };
 
 static ScratchLayout scratch_layout(int S, int64_t count, int64_t T) {
@@ -126,6 +126,7 @@ static ScratchLayout scratch_layout(int S, int64_t count, int64_t T) {
     L.qdone = off; off += (size_t)count * 4;          // qdone, work and qprog are contiguous:
     off = (off + 7) & ~(size_t)7;                     // one memset clears them
     L.work = off; off += 8;
+    L.cancel = off; off += 8;                         // u32 terminate flag (streaming)
     L.qprog = off; off = align256(off + (size_t)T * 4);  // <= T quanta
     L.total = off;
     return L;
@@ -533,6 +534,8 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     P.st_qdone = (unsigned int*)(sc + L.qdone);
     P.work = (unsigned long long*)(sc + L.work);
     P.qprog = m->stream ? (unsigned int*)(sc + L.qprog) : nullptr;
+    P.cancel = m->stream ? (const unsigned int*)(sc + L.cancel) : nullptr;
+    m->cancel_requested = false;
     P.logtab = m->d_logtab;
     P.smem_stats = dyn_smem ? 1 : 0;
 
@@ -583,6 +586,7 @@ static double quantile_from_hist(const int64_t* h, int B, int64_t n, double q, i
 }
 
 static void derive(cwc_model* m);
+static int64_t final_cuts(cwc_model* m, int64_t* items_done);
 
 void finalize(cwc_model* m, const int64_t* host_stats) {
     NvtxRange nvtx_range("cwc_stats_finalize");
@@ -595,6 +599,7 @@ void finalize(cwc_model* m, const int64_t* host_stats) {
     if (host_stats) std::memcpy(m->h_stats.data(), host_stats, len * 8);
     else ck(cudaMemcpy(m->h_stats.data(), m->d_stats, len * 8, cudaMemcpyDeviceToHost), "copy stats");
     m->cuts_final = m->K + 1;
+    if (m->cancel_requested && !host_stats) m->cuts_final = final_cuts(m, nullptr);
     derive(m);
     {   // reactions per recorded cut of this run (choose_fast_cut of the next simulation)
         int64_t recs = 0;
@@ -610,10 +615,9 @@ void finalize(cwc_model* m, const int64_t* host_stats) {
 // a separate stream.  Cuts below (q+1)*qs are final once every item of quanta 0..q has finished
 // (an instance that ended early emitted or filled all its later cuts).  The counters are read
 // before the statistics, so the snapshot contains every update of the cuts it reports final.
-void snapshot(cwc_model* m, int64_t* cuts_final, int64_t* items_done) {
-    NvtxRange nvtx_range("cwc_stats_snapshot");
-    if (!m->simulated) fail(CWC_E_STATE, "no simulation");
-    if (!m->stream) fail(CWC_E_STATE, "snapshots need the \"stream\" option set before simulating");
+// Cuts [0, result) are final: every item of quanta 0..q-1 has finished (from the progress
+// counters; stream option).  *items_done = finished items of all quanta.
+static int64_t final_cuts(cwc_model* m, int64_t* items_done) {
     if (!m->poll_stream) ck(cudaStreamCreateWithFlags(&m->poll_stream, cudaStreamNonBlocking), "cudaStreamCreate");
     const int64_t T = m->K + 1, nq = (T + m->qs - 1) / m->qs;
     const ScratchLayout L = scratch_layout(m->fm.S(), m->count, T);
@@ -624,11 +628,47 @@ void snapshot(cwc_model* m, int64_t* cuts_final, int64_t* items_done) {
     int64_t q = 0, done = 0;
     while (q < nq && prog[q] >= (uint64_t)m->count) ++q;
     for (uint32_t v : prog) done += v;
+    if (items_done) *items_done = done;
+    return std::min<int64_t>(q * m->qs, T);
+}
+
+// Terminate the running simulation (Fig. 2: "steer and terminate running
+// simulations"): the kernel stops handing out work items; items in flight finish their quantum,
+// so the cuts the progress counters report final stay exact.  Returns without waiting.
+void cancel(cwc_model* m) {
+    if (!m->simulated) fail(CWC_E_STATE, "no simulation");
+    if (!m->stream) fail(CWC_E_STATE, "cwc_cancel needs the \"stream\" option set before simulating");
+    if (!m->poll_stream) ck(cudaStreamCreateWithFlags(&m->poll_stream, cudaStreamNonBlocking), "cudaStreamCreate");
+    static const uint32_t one = 1;
+    const ScratchLayout L = scratch_layout(m->fm.S(), m->count, m->K + 1);
+    ck(cudaMemcpyAsync((char*)m->d_scratch + L.cancel, &one, 4, cudaMemcpyHostToDevice, m->poll_stream),
+       "set cancel flag");
+    ck(cudaStreamSynchronize(m->poll_stream), "set cancel flag");
+    m->cancel_requested = true;
+}
+
+// Replace the host statistics by a packed buffer of this geometry — e.g. the snapshots of all
+// ranks summed while their kernels run — and derive the views; no device synchronisation.
+void load_host_stats(cwc_model* m, const int64_t* host_stats, int64_t cuts_final) {
+    if (!m->simulated) fail(CWC_E_STATE, "no simulation");
+    if (!host_stats) fail(CWC_E_INVALID, "null statistics");
+    if (cuts_final < 0 || cuts_final > m->K + 1) fail(CWC_E_INVALID, "cuts_final outside [0, T]");
+    m->h_stats.assign(host_stats, host_stats + m->last_stats_len);
+    m->cuts_final = cuts_final;
+    derive(m);
+}
+
+void snapshot(cwc_model* m, int64_t* cuts_final, int64_t* items_done) {
+    NvtxRange nvtx_range("cwc_stats_snapshot");
+    if (!m->simulated) fail(CWC_E_STATE, "no simulation");
+    if (!m->stream) fail(CWC_E_STATE, "snapshots need the \"stream\" option set before simulating");
+    int64_t done = 0;
+    const int64_t cf = final_cuts(m, &done);   // counters first: the stats copy then holds them
     m->h_stats.resize(m->last_stats_len);
     ck(cudaMemcpyAsync(m->h_stats.data(), m->d_stats, m->last_stats_len * 8, cudaMemcpyDeviceToHost, m->poll_stream),
        "copy stats");
     ck(cudaStreamSynchronize(m->poll_stream), "copy stats");
-    m->cuts_final = std::min<int64_t>(q * m->qs, T);
+    m->cuts_final = cf;
     derive(m);
     if (cuts_final) *cuts_final = m->cuts_final;
     if (items_done) *items_done = done;

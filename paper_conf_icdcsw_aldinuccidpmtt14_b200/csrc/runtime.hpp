@@ -43,6 +43,7 @@ struct cwc_model {
     int64_t period_lo = 0, period_hi = 1;
     int period_window = 1;
     int stream = 0;                       // on-line streaming: progress counters + snapshots
+    bool cancel_requested = false;        // cwc_cancel on the running simulation
     cudaStream_t poll_stream = nullptr;   // copy-engine stream for snapshots
     int64_t cuts_final = 0;               // cuts final in the host views (T after finalize)
     int blocks_per_sm = 0;
@@ -108,6 +109,8 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
                     uint64_t seed, cudaStream_t stream, bool own_stream = false);
 void finalize(cwc_model* m, const int64_t* host_stats);
 void snapshot(cwc_model* m, int64_t* cuts_final, int64_t* items_done);
+void cancel(cwc_model* m);
+void load_host_stats(cwc_model* m, const int64_t* host_stats, int64_t cuts_final);
 void bind_buffers(cwc_model* m, int64_t* stats, size_t stats_n, int32_t* raw, size_t raw_n, void* scratch,
                   size_t scratch_bytes);
 void copy_samples(cwc_model* m, int64_t first, int64_t count, int32_t* out);

@@ -67,6 +67,33 @@ def simulate_sharded(model, n_total: int, t_end: float, sample_dt: float, seed: 
     return run.result()
 
 
+def combine_partial(packed, cuts_final: int, group=None):
+    """SUM the packed statistics and MIN the final-cut prefixes across ranks (host numpy in,
+    host numpy out): the combination rule of on-line multi-GPU streaming."""
+    import numpy as np
+    import torch
+    import torch.distributed as dist
+    buf = torch.from_numpy(np.ascontiguousarray(packed, dtype=np.int64).copy())
+    cf = torch.tensor([int(cuts_final)], dtype=torch.int64)
+    if dist.is_available() and dist.is_initialized() and dist.get_world_size(group) > 1:
+        if dist.get_backend(group) == "nccl":
+            buf, cf = buf.cuda(), cf.cuda()
+        dist.all_reduce(buf, op=dist.ReduceOp.SUM, group=group)
+        dist.all_reduce(cf, op=dist.ReduceOp.MIN, group=group)
+    return buf.cpu().numpy(), int(cf.cpu()[0])
+
+
+def snapshot_sharded(model, group=None):
+    """On-line streaming over ranks: every rank snapshots its own
+    running shard (copy engine, no synchronisation with its kernel), the packed statistics are
+    summed and the final-cut prefixes min-reduced across ranks, and the combined partial result is
+    loaded into ``model``.  Returns (cuts_final, EnsembleResult); cuts below cuts_final are the
+    whole ensemble's exact statistics.  Collective: call it on every rank."""
+    cf, _, _ = model.snapshot()
+    packed, cf_all = combine_partial(model.stats_host(), cf, group)
+    return cf_all, model.stats_load(packed, cf_all)
+
+
 def reduce_host_stats(local_stats, group=None):
     """Host-side combine used by CPU (gloo) tests: SUM-all-reduce a numpy int64 buffer."""
     import numpy as np

@@ -351,3 +351,33 @@ def test_streaming_snapshots_are_final_prefixes():
         n, t_end, cfg.sample_dt, cfg.seed)
     for name in ("n", "sum", "sqlo", "sqhi", "hist"):
         assert np.array_equal(getattr(ref, name), getattr(final, name))
+
+
+def test_stream_terminate_keeps_final_cuts_exact():
+    """Terminating a running simulation (Fig. 2; cwc_cancel via stream(stop=)):
+    the kernel stops early, and the cuts reported final are exactly the uninterrupted run's."""
+    import paper_conf_icdcsw_aldinuccidpmtt14_b200 as cwc
+    cfg = W.CONFIGS["schlogl"]
+    n = cfg.n_instances
+    m = cwc.Model.from_def(cfg.model, hist_bins=cfg.hist_bins, raw_samples=False)
+    out = list(m.stream(n, cfg.t_end, cfg.sample_dt, cfg.seed, poll_s=0.002, stop=lambda cf, res: cf > 0))
+    cf, res = out[-1]
+    T = res.n.size
+    assert 0 < cf < T, [c for c, _ in out]          # stopped after the first final cuts, well before T
+    ref = cwc.Model.from_def(cfg.model, hist_bins=cfg.hist_bins, raw_samples=False).simulate(
+        n, cfg.t_end, cfg.sample_dt, cfg.seed)
+    assert res.reactions < ref.reactions // 2       # most of the work was not done
+    for name in ("n", "sum", "sqlo", "sqhi", "hist"):
+        assert np.array_equal(getattr(res, name)[:cf], getattr(ref, name)[:cf]), name
+    assert (res.n[:cf] == n).all() and (res.n[cf:] < n).any()
+    # a new simulation on the same handle is unaffected by the earlier terminate
+    again = m.simulate(1000, 5.0, cfg.sample_dt, cfg.seed)
+    assert again.finished == 1000
+
+
+def test_cancel_needs_streaming():
+    import paper_conf_icdcsw_aldinuccidpmtt14_b200 as cwc
+    m = cwc.Model.from_def(W.IMM_DEATH, hist_bins=64)
+    m.simulate(100, 10.0, 1.0, 1)
+    with pytest.raises(cwc.CWCError):
+        m.cancel()

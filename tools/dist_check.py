@@ -42,6 +42,30 @@ def main():
         for name in ("n", "sum", "sqlo", "sqhi", "hist"):
             ok &= bool(np.array_equal(getattr(res, name), getattr(ref, name)))
         ok &= res.reactions == ref.reactions and res.finished == N
+    # on-line streaming across ranks (dist.snapshot_sharded): combined partial results while the
+    # shards run; the final-cut prefix of every combined snapshot equals the whole run's
+    import time
+    from paper_conf_icdcsw_aldinuccidpmtt14_b200.dist import shard, snapshot_sharded
+    N2, t2 = 100_000, 10.0
+    first, count = shard(N2, rank, world)
+    m2 = cwc.Model.from_def(md, hist_bins=512, device=local, raw_samples=False, stream=1)
+    m2.simulate_range(N2, first, count, t2, dt, seed)
+    T2 = int(round(t2 / dt)) + 1
+    snaps = []
+    while True:
+        cf, r2 = snapshot_sharded(m2)          # collective: same cf on every rank
+        snaps.append((cf, {k: getattr(r2, k).copy() for k in ("n", "sum", "sqlo", "sqhi", "hist")}))
+        if cf >= T2:
+            break
+        time.sleep(0.005)
+    m2.finalize()
+    if rank == 0:
+        ref2 = cwc.Model.from_def(md, hist_bins=512, device=local, raw_samples=False).simulate(N2, t2, dt, seed)
+        for cf, st in snaps:
+            for name, v in st.items():
+                ok &= bool(np.array_equal(v[:cf], getattr(ref2, name)[:cf]))
+        partial = sorted({cf for cf, _ in snaps if 0 < cf < T2})
+        print(f"streamed snapshots: final prefixes {partial[:8]}... of T={T2}", flush=True)
         print(("DIST OK" if ok else "DIST MISMATCH") + f" world={world} backend={backend} reactions={res.reactions}",
               flush=True)
     dist.barrier()
