@@ -20,6 +20,7 @@ def main():
     runs = [
         (W.IMM_DEATH, 300, 10.0, 1.0, {}),
         (W.LOTKA_VOLTERRA, 300, 0.3, 0.05, {"quantum_samples": 2}),
+        (W.LOTKA_VOLTERRA, 300, 0.3, 0.05, {"fast_cut": 1}),
         (W.SCHLOGL, 500, 0.5, 0.05, {"quantum_samples": 2, "block_threads": 128}),
         (W.CIRCADIAN, 200, 4.0, 0.5, {"period_species": "R", "period_lo": 100, "period_hi": 1000}),
         (W.COMPARTMENTS, 200, 2.0, 0.5, {"smem_stats": 0}),
@@ -38,6 +39,15 @@ def main():
     for cf, res in m.stream(2000, 0.5, 0.05, 7, poll_s=0.001):
         pass
     print("stream ok", flush=True)
+    # terminate mid-run (cwc_cancel) and the LV path with cuts recorded outside the fast step
+    m = cwc.Model.from_def(W.SCHLOGL, hist_bins=64, raw_samples=False)
+    for cf, res in m.stream(4000, 1.0, 0.05, 9, poll_s=0.001, stop=lambda c, r: c > 0):
+        pass
+    print(f"cancel ok (cuts final {cf})", flush=True)
+    m = cwc.Model.from_def(W.VESICLES, hist_bins=64, quantum_samples=3)
+    res = m.simulate(300, 3.0, 0.5, 5)
+    assert res.finished == 300
+    print("vesicles (dynamic pools) ok", flush=True)
 
 
 if __name__ == "__main__":
