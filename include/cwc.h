@@ -267,6 +267,24 @@ cwc_status cwc_stats_snapshot(cwc_model_t m, int64_t* cuts_final, int64_t* items
  * statistics are exact; later cuts are partial).  Errors: CWC_E_STATE without a streaming
  * simulation. */
 cwc_status cwc_cancel(cwc_model_t m);
+
+/* Checkpoint / resume (the paper's tasks are resumable at quantum boundaries,
+ * P:L241-243).  Because the RNG is counter-based (R3), the per-instance records (x, t, step, k,
+ * flags, period state) and the quanta each instance has done are a complete checkpoint: a resumed
+ * run is bit-identical to the uninterrupted one.
+ *   cwc_checkpoint_bytes / _save: after the last simulation's kernel has finished (it synchronises)
+ *     — statistics, instance records, queue state and raw cuts into a caller-owned host buffer.
+ *   cwc_checkpoint_load: into a handle of the same model and result-affecting options (flat
+ *     network, histogram, x_cap, raw_samples, period analysis — checked by hash); the run can
+ *     then be continued or finalised as it stands.
+ *   cwc_resume: continue a run ended by cwc_cancel, or restored, to its horizon on cuda_stream
+ *     (NULL = legacy default stream; asynchronous); quanta already done are skipped.
+ * Errors: CWC_E_STATE (nothing simulated / nothing to resume), CWC_E_INVALID (buffer too small,
+ * not a checkpoint, other model or geometry), CWC_E_CUDA. */
+cwc_status cwc_checkpoint_bytes(cwc_model_t m, size_t* bytes);
+cwc_status cwc_checkpoint_save(cwc_model_t m, void* out, size_t bytes);
+cwc_status cwc_checkpoint_load(cwc_model_t m, const void* in, size_t bytes);
+cwc_status cwc_resume(cwc_model_t m, void* cuda_stream);
 /* The packed statistics (layout above) behind the current cwc_stats views, as copied by the last
  * snapshot or finalize: a borrowed host view valid until the next snapshot / finalize / load /
  * simulate / free.  CWC_E_STATE before the first snapshot or finalize. */

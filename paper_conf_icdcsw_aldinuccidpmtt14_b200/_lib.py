@@ -74,6 +74,10 @@ SIGNATURES = {
     "cwc_kernel_attributes": (c_i32, [c_vp, P(c_i32), P(c_i32), P(c_i32)]),
     "cwc_kernel_image": (c_i32, [c_vp, P(c_vp), P(c_sz)]),
     "cwc_cancel": (c_i32, [c_vp]),
+    "cwc_resume": (c_i32, [c_vp, c_vp]),
+    "cwc_checkpoint_bytes": (c_i32, [c_vp, P(c_sz)]),
+    "cwc_checkpoint_save": (c_i32, [c_vp, c_vp, c_sz]),
+    "cwc_checkpoint_load": (c_i32, [c_vp, c_vp, c_sz]),
     "cwc_stats_host": (c_i32, [c_vp, P(c_vp), P(c_sz)]),
     "cwc_stats_load": (c_i32, [c_vp, c_vp, c_i64]),
     "cwc_buffer_sizes": (c_i32, [c_vp, c_i64, c_dbl, c_dbl, P(c_sz), P(c_sz), P(c_sz)]),

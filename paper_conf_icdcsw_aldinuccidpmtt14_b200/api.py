@@ -266,6 +266,28 @@ class Model:
         check(lib.cwc_stats_load(self._h, _ptr(buf), int(cuts_final)))
         return self.stats()
 
+    def checkpoint(self) -> np.ndarray:
+        """The last simulation as a host checkpoint (cwc_checkpoint_save; synchronises)."""
+        n = ctypes.c_size_t()
+        check(lib.cwc_checkpoint_bytes(self._h, ctypes.byref(n)))
+        buf = np.empty(n.value, dtype=np.uint8)
+        check(lib.cwc_checkpoint_save(self._h, _ptr(buf), n.value))
+        return buf
+
+    def restore(self, ckpt: np.ndarray) -> None:
+        """Load a checkpoint of the same model / options into this handle (cwc_checkpoint_load)."""
+        buf = np.ascontiguousarray(ckpt, dtype=np.uint8)
+        check(lib.cwc_checkpoint_load(self._h, _ptr(buf), buf.size))
+
+    def resume(self, stream=None) -> None:
+        """Continue a terminated or restored run to its horizon (cwc_resume; asynchronous)."""
+        if stream is None:
+            import torch
+            stream = torch.cuda.current_stream()
+        if hasattr(stream, "cuda_stream"):
+            stream = stream.cuda_stream
+        check(lib.cwc_resume(self._h, ctypes.c_void_p(int(stream) if stream else 0)))
+
     def cancel(self):
         """Terminate the running streaming simulation (cwc_cancel)."""
         check(lib.cwc_cancel(self._h))

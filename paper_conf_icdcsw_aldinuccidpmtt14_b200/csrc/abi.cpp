@@ -386,6 +386,34 @@ cwc_status cwc_stats_load(cwc_model_t m, const int64_t* host_stats, int64_t cuts
     });
 }
 
+cwc_status cwc_resume(cwc_model_t m, void* cuda_stream) {
+    return guard([&] {
+        need(m != nullptr, "NULL model");
+        cwc::resume(m, (cudaStream_t)cuda_stream);
+    });
+}
+
+cwc_status cwc_checkpoint_bytes(cwc_model_t m, size_t* bytes) {
+    return guard([&] {
+        need(m != nullptr && bytes != nullptr, "bad arguments");
+        *bytes = cwc::checkpoint_bytes(m);
+    });
+}
+
+cwc_status cwc_checkpoint_save(cwc_model_t m, void* out, size_t bytes) {
+    return guard([&] {
+        need(m != nullptr, "NULL model");
+        cwc::checkpoint_save(m, out, bytes);
+    });
+}
+
+cwc_status cwc_checkpoint_load(cwc_model_t m, const void* in, size_t bytes) {
+    return guard([&] {
+        need(m != nullptr, "NULL model");
+        cwc::checkpoint_load(m, in, bytes);
+    });
+}
+
 cwc_status cwc_cancel(cwc_model_t m) {
     return guard([&] {
         need(m != nullptr, "NULL model");

@@ -20,7 +20,7 @@ struct cwc_params {
     long long n_items;          // work items = n_quanta * count
     long long qs;               // cuts per quantum (Q/tau)
     int refill;                 // 1 = global atomic work queue with warp-aggregated refill
-    int pad0;
+    int resume;                 // 1: continue a terminated / restored run (skip quanta already done)
     cwc_round_keys rk;          // Philox round keys of the seed
     unsigned long long* stats;  // packed int64 stats (cwc.h layout)
     int* raw;                   // [ceil(T/8)][S][count][8] (time-blocked SoA) or nullptr

@@ -432,7 +432,7 @@ static bool choose_fast_cut(cwc_model* m, double dt) {
 }
 
 void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count, double t_end, double dt,
-                    uint64_t seed, cudaStream_t stream, bool own_stream) {
+                    uint64_t seed, cudaStream_t stream, bool own_stream, bool resume) {
     NvtxRange nvtx_range("cwc_simulate_range");
     if (n_total <= 0) fail(CWC_E_INVALID, "n_total must be > 0");
     if (first < 0 || count < 0 || first + count > n_total) fail(CWC_E_INVALID, "instance range outside [0, n_total)");
@@ -505,6 +505,7 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     else if (m->quantum_samples > 0) qs = std::min<int64_t>(m->quantum_samples, T);
     else if (m->stream) qs = std::max<int64_t>(1, (T + 15) / 16);  // streaming: progress in ~16 chunks
     else qs = (count >= 4 * lanes) ? (T + 7) / 8 : T;
+    if (resume) qs = m->qs;  // the work items (quantum, instance) of the run being continued
     const int64_t nq = (T + qs - 1) / qs;
 
     const ScratchLayout L = scratch_layout(S, count, T);
@@ -518,6 +519,7 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     P.n_items = nq * count;
     P.qs = qs;
     P.refill = m->refill;
+    P.resume = resume ? 1 : 0;
     const uint32_t key0 = (uint32_t)seed, key1 = (uint32_t)(seed >> 32);
     for (int r = 0; r < 10; ++r) {
         P.rk.k0[r] = key0 + (uint32_t)r * 0x9E3779B9u;
@@ -539,8 +541,13 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     P.logtab = m->d_logtab;
     P.smem_stats = dyn_smem ? 1 : 0;
 
-    ck(cudaMemsetAsync(m->d_stats, 0, need_stats * 8, stream), "memset(stats)");
-    ck(cudaMemsetAsync(sc + L.qdone, 0, L.qprog + (size_t)T * 4 - L.qdone, stream), "memset(queue)");
+    if (!resume) {
+        ck(cudaMemsetAsync(m->d_stats, 0, need_stats * 8, stream), "memset(stats)");
+        ck(cudaMemsetAsync(sc + L.qdone, 0, L.qprog + (size_t)T * 4 - L.qdone, stream), "memset(queue)");
+    } else {  // keep statistics, instance states, quanta done and progress; restart the hand-out
+        ck(cudaMemsetAsync(sc + L.work, 0, L.qprog - L.work, stream), "memset(work, cancel)");
+    }
+    m->resumable = false;
     ck(cudaEventRecord(m->ev0, stream), "cudaEventRecord");
     if (count > 0) {
         void* args[] = {&P};
@@ -645,6 +652,7 @@ void cancel(cwc_model* m) {
        "set cancel flag");
     ck(cudaStreamSynchronize(m->poll_stream), "set cancel flag");
     m->cancel_requested = true;
+    m->resumable = true;
 }
 
 // Replace the host statistics by a packed buffer of this geometry — e.g. the snapshots of all
@@ -656,6 +664,132 @@ void load_host_stats(cwc_model* m, const int64_t* host_stats, int64_t cuts_final
     m->h_stats.assign(host_stats, host_stats + m->last_stats_len);
     m->cuts_final = cuts_final;
     derive(m);
+}
+
+// ------------------------------------------------------------------------ checkpoint / resume
+// the counter-based RNG makes the per-instance record (x, t, step, k, flags, period
+// state) plus the quanta done a complete checkpoint — a continued run draws exactly the numbers
+// the uninterrupted one would have (R3), so resuming is bit-identical.
+
+// What a checkpoint must agree with: the flat model and every option that changes results.
+static uint64_t model_identity(const cwc_model* m) {
+    std::ostringstream o;
+    const FlatModel& f = m->fm;
+    char buf[40];
+    for (const auto& n : f.names) o << n << ';';
+    for (int32_t v : f.x0) o << v << ',';
+    for (double r : f.rates) { std::snprintf(buf, sizeof buf, "%a,", r); o << buf; }
+    for (const auto& rl : f.reactants) { for (const auto& r : rl) o << r.species << ':' << r.order << ' '; o << '|'; }
+    for (const auto& d : f.delta) { for (int32_t v : d) o << v << ','; o << '|'; }
+    for (size_t j = 0; j < f.law.size(); ++j) {
+        std::snprintf(buf, sizeof buf, "%a", f.law_K[j]);
+        o << f.law[j] << ':' << f.law_species[j] << ':' << f.law_n[j] << ':' << buf << ';';
+    }
+    for (size_t j = 0; j < f.gate_species.size(); ++j) o << f.gate_species[j] << ':' << f.gate_kind[j] << ';';
+    for (const auto& pl : f.place)
+        for (const auto& sl : pl) { o << sl.alive << '<'; for (const auto& a : sl.adds) o << a.first << '+' << a.second << ' '; }
+    for (const auto& tr : f.transfer) for (const auto& t : tr) o << t.first << '>' << t.second << ' ';
+    o << '#' << f.sentinel << ';' << m->hist_bins << ';' << m->x_cap << ';' << m->raw_samples << ';'
+      << m->period_species << ';' << m->period_lo << ';' << m->period_hi << ';';
+    for (size_t s = 0; s < m->hist_lo.size(); ++s) o << m->hist_lo[s] << '/' << m->hist_width[s] << ',';
+    return fnv1a(o.str());
+}
+
+namespace {
+struct CkptHeader {
+    char magic[8];
+    uint64_t identity;
+    int64_t n_total, first, count, K, qs;
+    double dt, t_end;
+    uint64_t seed;
+    uint64_t stats_len, raw_len, scratch_bytes;
+};
+const char kCkptMagic[8] = {'C', 'W', 'C', 'C', 'K', 'P', 'T', '1'};
+}  // namespace
+
+size_t checkpoint_bytes(cwc_model* m) {
+    if (!m->simulated) fail(CWC_E_STATE, "no simulation to checkpoint");
+    size_t ns, nr, nsc;
+    buffer_sizes(m, m->count, m->K, &ns, &nr, &nsc);
+    return sizeof(CkptHeader) + ns * 8 + nsc + nr * 4;
+}
+
+// After the kernel has finished (a completed or terminated run): header, statistics, instance
+// records + queue state, raw cuts.
+void checkpoint_save(cwc_model* m, void* out, size_t bytes) {
+    const size_t need = checkpoint_bytes(m);
+    if (!out || bytes < need) fail(CWC_E_INVALID, "checkpoint buffer too small (see cwc_checkpoint_bytes)");
+    ck(cudaStreamSynchronize(m->last_stream), "simulation");
+    CkptHeader h{};
+    std::memcpy(h.magic, kCkptMagic, 8);
+    h.identity = model_identity(m);
+    h.n_total = m->n_total; h.first = m->first; h.count = m->count; h.K = m->K; h.qs = m->qs;
+    h.dt = m->dt; h.t_end = m->t_end; h.seed = m->seed;
+    size_t ns, nr, nsc;
+    buffer_sizes(m, m->count, m->K, &ns, &nr, &nsc);
+    h.stats_len = ns; h.raw_len = nr; h.scratch_bytes = nsc;
+    char* p = (char*)out;
+    std::memcpy(p, &h, sizeof h);
+    p += sizeof h;
+    ck(cudaMemcpy(p, m->d_stats, ns * 8, cudaMemcpyDeviceToHost), "checkpoint stats");
+    p += ns * 8;
+    ck(cudaMemcpy(p, m->d_scratch, nsc, cudaMemcpyDeviceToHost), "checkpoint scratch");
+    p += nsc;
+    if (nr) ck(cudaMemcpy(p, m->d_raw, nr * 4, cudaMemcpyDeviceToHost), "checkpoint raw");
+}
+
+// Restore a checkpoint into this handle (same model and result-affecting options); the run can
+// then be continued with cwc_resume or finalised as it stands.
+void checkpoint_load(cwc_model* m, const void* in, size_t bytes) {
+    if (!in || bytes < sizeof(CkptHeader)) fail(CWC_E_INVALID, "not a checkpoint");
+    CkptHeader h;
+    std::memcpy(&h, in, sizeof h);
+    if (std::memcmp(h.magic, kCkptMagic, 8) != 0) fail(CWC_E_INVALID, "not a checkpoint");
+    if (h.identity != model_identity(m)) fail(CWC_E_INVALID, "checkpoint of a different model or options");
+    size_t ns, nr, nsc;
+    buffer_sizes(m, h.count, h.K, &ns, &nr, &nsc);
+    if (ns != h.stats_len || nr != h.raw_len || nsc != h.scratch_bytes ||
+        bytes < sizeof h + ns * 8 + nsc + nr * 4)
+        fail(CWC_E_INVALID, "checkpoint geometry does not match the model's buffers");
+    const int dev = current_device(m);
+    ck(cudaSetDevice(dev), "cudaSetDevice");
+    if (m->bound) {
+        if (m->stats_cap < ns * 8 || m->scratch_cap < nsc || (nr && m->raw_cap < nr * 4))
+            fail(CWC_E_INVALID, "bound device buffers too small for the checkpoint");
+    } else {
+        grow(m->d_stats, m->stats_cap, ns * 8, "cudaMalloc(stats)");
+        if (nr) grow(m->d_raw, m->raw_cap, nr * 4, "cudaMalloc(raw)");
+        grow(m->d_scratch, m->scratch_cap, nsc, "cudaMalloc(scratch)");
+    }
+    const char* p = (const char*)in + sizeof h;
+    ck(cudaMemcpy(m->d_stats, p, ns * 8, cudaMemcpyHostToDevice), "restore stats");
+    p += ns * 8;
+    ck(cudaMemcpy(m->d_scratch, p, nsc, cudaMemcpyHostToDevice), "restore scratch");
+    p += nsc;
+    if (nr) ck(cudaMemcpy(m->d_raw, p, nr * 4, cudaMemcpyHostToDevice), "restore raw");
+    if (!m->ev0) {
+        ck(cudaEventCreate(&m->ev0), "cudaEventCreate");
+        ck(cudaEventCreate(&m->ev1), "cudaEventCreate");
+    }
+    ck(cudaEventRecord(m->ev0, nullptr), "cudaEventRecord");
+    ck(cudaEventRecord(m->ev1, nullptr), "cudaEventRecord");
+    m->simulated = true;
+    m->finalized = false;
+    m->last_stream = nullptr;
+    m->n_total = h.n_total; m->first = h.first; m->count = h.count; m->K = h.K; m->qs = h.qs;
+    m->dt = h.dt; m->t_end = h.t_end; m->seed = h.seed;
+    m->last_stats_len = ns;
+    m->items = ((h.K + 1 + h.qs - 1) / h.qs) * h.count;
+    m->cancel_requested = false;
+    m->resumable = true;
+}
+
+// Continue a terminated or restored run to its horizon on `stream` (asynchronous, like
+// simulate_range): quanta already done are skipped, statistics keep accumulating.
+void resume(cwc_model* m, cudaStream_t stream) {
+    if (!m->simulated || !m->resumable) fail(CWC_E_STATE, "nothing to resume (terminate or restore a run first)");
+    ck(cudaStreamSynchronize(m->last_stream), "terminated simulation");
+    simulate_range(m, m->n_total, m->first, m->count, m->t_end, m->dt, m->seed, stream, false, true);
 }
 
 void snapshot(cwc_model* m, int64_t* cuts_final, int64_t* items_done) {

@@ -44,6 +44,7 @@ struct cwc_model {
     int period_window = 1;
     int stream = 0;                       // on-line streaming: progress counters + snapshots
     bool cancel_requested = false;        // cwc_cancel on the running simulation
+    bool resumable = false;               // terminated (or restored) run that cwc_resume can continue
     cudaStream_t poll_stream = nullptr;   // copy-engine stream for snapshots
     int64_t cuts_final = 0;               // cuts final in the host views (T after finalize)
     int blocks_per_sm = 0;
@@ -106,7 +107,11 @@ size_t stats_len(int64_t T, int S, int B, bool period);
 void buffer_sizes(const cwc_model* m, int64_t count, int64_t K, size_t* stats, size_t* raw, size_t* scratch);
 void compile(cwc_model* m, const uint64_t* seed = nullptr);  // NVRTC (no GPU needed)
 void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count, double t_end, double dt,
-                    uint64_t seed, cudaStream_t stream, bool own_stream = false);
+                    uint64_t seed, cudaStream_t stream, bool own_stream = false, bool resume = false);
+void resume(cwc_model* m, cudaStream_t stream);
+size_t checkpoint_bytes(cwc_model* m);
+void checkpoint_save(cwc_model* m, void* out, size_t bytes);
+void checkpoint_load(cwc_model* m, const void* in, size_t bytes);
 void finalize(cwc_model* m, const int64_t* host_stats);
 void snapshot(cwc_model* m, int64_t* cuts_final, int64_t* items_done);
 void cancel(cwc_model* m);

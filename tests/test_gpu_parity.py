@@ -381,3 +381,53 @@ def test_cancel_needs_streaming():
     m.simulate(100, 10.0, 1.0, 1)
     with pytest.raises(cwc.CWCError):
         m.cancel()
+
+
+def test_checkpoint_resume_bit_identical():
+    """Terminate a running simulation, checkpoint it to the host, restore it into a fresh handle
+    and resume it: statistics, raw cuts and per-instance records equal the uninterrupted run
+    (counter-based RNG); resuming on the same handle gives the same."""
+    import paper_conf_icdcsw_aldinuccidpmtt14_b200 as cwc
+    cfg = W.CONFIGS["schlogl"]
+    n, t_end = 200_000, 20.0
+    kw = dict(hist_bins=cfg.hist_bins, quantiles=QS)
+    ref_m = cwc.Model.from_def(cfg.model, **kw)
+    ref = ref_m.simulate(n, t_end, cfg.sample_dt, cfg.seed)
+    ref_raw = ref_m.samples(0, n)
+    ref_flags, ref_react, _ = ref_m.records(0, n)
+
+    m = cwc.Model.from_def(cfg.model, **kw)
+    out = list(m.stream(n, t_end, cfg.sample_dt, cfg.seed, poll_s=0.002, stop=lambda cf, r: cf > 0))
+    cf, part = out[-1]
+    assert 0 < cf < part.n.size and part.reactions < ref.reactions
+    ckpt = m.checkpoint()
+
+    m2 = cwc.Model.from_def(cfg.model, **kw)
+    m2.restore(ckpt)
+    m2.resume()
+    for mm in (m2, m):
+        if mm is m:
+            m.resume()
+        res = mm.finalize()
+        for name in ("n", "sum", "sqlo", "sqhi", "hist", "quantile"):
+            assert np.array_equal(getattr(res, name), getattr(ref, name), equal_nan=True), name
+        assert res.reactions == ref.reactions and res.finished == n and res.absorbed == ref.absorbed
+        assert np.array_equal(mm.samples(0, n), ref_raw)
+        flags, react, _ = mm.records(0, n)
+        assert np.array_equal(flags, ref_flags) and np.array_equal(react, ref_react)
+
+
+def test_checkpoint_rejects_other_model_and_nothing_to_resume():
+    import paper_conf_icdcsw_aldinuccidpmtt14_b200 as cwc
+    m = cwc.Model.from_def(W.IMM_DEATH, hist_bins=64)
+    m.simulate(100, 10.0, 1.0, 1)
+    ckpt = m.checkpoint()
+    with pytest.raises(cwc.CWCError):
+        m.resume()                                  # a completed run: nothing to resume
+    other = cwc.Model.from_def(W.IMM_DEATH, hist_bins=65)
+    with pytest.raises(cwc.CWCError):
+        other.restore(ckpt)                         # different histogram: different results
+    same = cwc.Model.from_def(W.IMM_DEATH, hist_bins=64)
+    same.restore(ckpt)                              # a finished run restores and finalises as is
+    res = same.finalize()
+    assert res.finished == 100 and np.array_equal(res.hist, m.finalize().hist)
