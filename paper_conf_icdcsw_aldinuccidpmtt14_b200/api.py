@@ -12,6 +12,7 @@ stream so the caller can time it with CUDA events and all-reduce the stats with 
 from __future__ import annotations
 
 import ctypes
+import weakref
 from dataclasses import dataclass
 from typing import List, Optional, Sequence
 
@@ -366,7 +367,9 @@ class DeviceBuffers:
         self.stats = torch.empty(n_stats, dtype=torch.int64, device=dev)
         self.raw = torch.empty(max(n_raw, 1), dtype=torch.int32, device=dev) if n_raw else None
         self.scratch = torch.empty(n_scratch, dtype=torch.uint8, device=dev)
-        self.model = model
+        # weak back-reference: the model holds its bound buffers (below), and a strong cycle would
+        # keep both alive until a garbage-collector pass (device memory not returned on del)
+        self._model = weakref.ref(model)
         model.set_option("device", dev.index)
         check(lib.cwc_bind_device_buffers(
             model.handle, ctypes.c_void_p(self.stats.data_ptr()), n_stats,
@@ -378,9 +381,16 @@ class DeviceBuffers:
         model._bound_buffers = self
 
     def unbind(self):
-        check(lib.cwc_bind_device_buffers(self.model.handle, None, 0, None, 0, None, 0))
-        if getattr(self.model, "_bound_buffers", None) is self:
-            self.model._bound_buffers = None
+        model = self._model()
+        if model is None or not model.handle:
+            return
+        check(lib.cwc_bind_device_buffers(model.handle, None, 0, None, 0, None, 0))
+        if getattr(model, "_bound_buffers", None) is self:
+            model._bound_buffers = None
+
+    @property
+    def model(self):
+        return self._model()
 
 
 def selftest_philox(ctr: np.ndarray, key: np.ndarray) -> np.ndarray:
