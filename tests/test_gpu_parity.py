@@ -431,3 +431,29 @@ def test_checkpoint_rejects_other_model_and_nothing_to_resume():
     same.restore(ckpt)                              # a finished run restores and finalises as is
     res = same.finalize()
     assert res.finished == 100 and np.array_equal(res.hist, m.finalize().hist)
+
+
+def test_checkpoint_resume_with_period_analysis():
+    """The on-line period detector's per-instance state travels in the checkpoint: a terminated,
+    restored and resumed circadian run gives the uninterrupted run's period statistics."""
+    import paper_conf_icdcsw_aldinuccidpmtt14_b200 as cwc
+    pa = W.PERIOD_ANALYSIS["circadian"]
+    n, t_end, dt, seed = 40_000, 96.0, 0.5, 17
+    kw = dict(hist_bins=64, raw_samples=False, period_species=pa["species"], period_lo=pa["lo"],
+              period_hi=pa["hi"], period_window=pa["window"])
+    ref_m = cwc.Model.from_def(W.CIRCADIAN, **kw)
+    ref = ref_m.simulate(n, t_end, dt, seed)
+    ref_p = ref_m.period_stats()
+    m = cwc.Model.from_def(W.CIRCADIAN, **kw)
+    cf, part = list(m.stream(n, t_end, dt, seed, poll_s=0.001, stop=lambda c, r: c > 0))[-1]
+    assert 0 < cf < part.n.size
+    m2 = cwc.Model.from_def(W.CIRCADIAN, **kw)
+    m2.restore(m.checkpoint())
+    m2.resume()
+    res = m2.finalize()
+    got = m2.period_stats()
+    for name in ("n", "sum", "sqlo", "sqhi", "hist"):
+        assert np.array_equal(getattr(res, name), getattr(ref, name)), name
+    for name in ("events", "pc_n", "pc_sum", "pc_sqlo", "pc_sqhi", "lp_n", "lp_sum", "lp_sqlo", "lp_sqhi"):
+        assert np.array_equal(got[name], ref_p[name]), name
+    assert np.array_equal(got["moving_avg"], ref_p["moving_avg"], equal_nan=True)
