@@ -230,8 +230,11 @@ def run_b200(args):
         with torch.cuda.stream(stream):
             flush.zero_()
         run.launch(cfg.seed + w, stream)
+        # finalise every warm-up run: the kernel variant (cut recording, runtime.cpp
+        # choose_fast_cut) adapts to the measured reactions per cut, and its NVRTC compile must
+        # happen here, not inside the first timed step
+        res = run.result()
     torch.cuda.synchronize()
-    res = run.result()
 
     clocks = ClockSampler(local)
     ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True),
