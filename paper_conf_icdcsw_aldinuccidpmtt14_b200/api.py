@@ -22,6 +22,17 @@ from . import _lib
 from ._lib import CWCError, check, lib  # noqa: F401
 
 
+def _stream_handle(stream):
+    """cudaStream_t of a torch.cuda.Stream / raw handle; None = torch's current stream (the legacy
+    default stream, 0, when CUDA is unavailable — the library then reports CWC_E_CUDA)."""
+    if stream is None:
+        import torch
+        stream = torch.cuda.current_stream() if torch.cuda.is_available() else 0
+    if hasattr(stream, "cuda_stream"):
+        stream = stream.cuda_stream
+    return int(stream) if stream else 0
+
+
 def _ptr(a: np.ndarray):
     return ctypes.c_void_p(a.ctypes.data)
 
@@ -211,13 +222,9 @@ class Model:
                        stream=None) -> None:
         """Enqueue instances [first, first+count) on ``stream``: a torch.cuda.Stream, a raw
         cudaStream_t int, or None for torch's current stream.  Asynchronous."""
-        if stream is None:
-            import torch
-            stream = torch.cuda.current_stream()
-        if hasattr(stream, "cuda_stream"):
-            stream = stream.cuda_stream
+        stream = _stream_handle(stream)
         check(lib.cwc_simulate_range(self._h, int(n_total), int(first), int(count), float(t_end),
-                                     float(sample_dt), int(seed), ctypes.c_void_p(int(stream))))
+                                     float(sample_dt), int(seed), ctypes.c_void_p(stream)))
 
     def finalize(self, host_stats: Optional[np.ndarray] = None) -> EnsembleResult:
         if host_stats is not None:
@@ -282,12 +289,8 @@ class Model:
 
     def resume(self, stream=None) -> None:
         """Continue a terminated or restored run to its horizon (cwc_resume; asynchronous)."""
-        if stream is None:
-            import torch
-            stream = torch.cuda.current_stream()
-        if hasattr(stream, "cuda_stream"):
-            stream = stream.cuda_stream
-        check(lib.cwc_resume(self._h, ctypes.c_void_p(int(stream) if stream else 0)))
+        stream = _stream_handle(stream)
+        check(lib.cwc_resume(self._h, ctypes.c_void_p(stream)))
 
     def cancel(self):
         """Terminate the running streaming simulation (cwc_cancel)."""

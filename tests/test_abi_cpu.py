@@ -190,3 +190,20 @@ def test_simulate_without_gpu_fails_loudly():
     with pytest.raises(cwc.CWCError) as e:
         m.simulate(10, 1.0, 1.0, 1)
     assert e.value.status == 4
+
+
+def test_steering_and_checkpoint_calls_out_of_order():
+    """Terminate / resume / checkpoint / host-stats calls before any simulation are state errors
+    (no device needed); a restore of garbage is rejected as invalid input."""
+    import numpy as np
+    m = cwc.Model.from_def(W.IMM_DEATH)
+    for call in (m.cancel, m.resume, m.checkpoint, m.stats_host):
+        with pytest.raises(cwc.CWCError) as e:
+            call()
+        assert e.value.status == 6, call
+    with pytest.raises(cwc.CWCError) as e:
+        m.stats_load(np.zeros(10, dtype=np.int64), 0)
+    assert e.value.status == 6
+    with pytest.raises(cwc.CWCError) as e:
+        m.restore(np.zeros(64, dtype=np.uint8))
+    assert e.value.status == 1
