@@ -576,20 +576,27 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
 }
 
 // ------------------------------------------------------------------------------------ finalize
-static double quantile_from_hist(const int64_t* h, int B, int64_t n, double q, int64_t lo, int64_t w) {
-    if (n == 0) return NAN;
-    int64_t need = (int64_t)std::ceil(q * (double)n);
-    if (need < 1) need = 1;
+// All quantile levels of one (cut, species) histogram in one scan (R11: the left edge of the
+// first bin whose cumulative count reaches max(1, ceil(q n)); under/overflow give -inf/+inf): `order` lists the level indices by increasing level.
+static void quantiles_from_hist(const int64_t* h, int B, int64_t n, const std::vector<double>& q,
+                                const std::vector<int>& order, int64_t lo, int64_t w, double* out) {
+    if (n == 0) {
+        for (size_t i = 0; i < q.size(); ++i) out[i] = NAN;
+        return;
+    }
+    size_t next = 0;
     int64_t c = 0;
-    for (int b = 0; b < B + 2; ++b) {
+    for (int b = 0; b < B + 2 && next < order.size(); ++b) {
         c += h[b];
-        if (c >= need) {
-            if (b == 0) return -INFINITY;
-            if (b == B + 1) return INFINITY;
-            return (double)(lo + w * (int64_t)(b - 1));
+        while (next < order.size()) {
+            int64_t need = (int64_t)std::ceil(q[order[next]] * (double)n);
+            if (need < 1) need = 1;
+            if (c < need) break;
+            out[order[next]] = b == 0 ? -INFINITY : (b == B + 1 ? INFINITY : (double)(lo + w * (int64_t)(b - 1)));
+            ++next;
         }
     }
-    return INFINITY;
+    for (; next < order.size(); ++next) out[order[next]] = INFINITY;
 }
 
 static void derive(cwc_model* m);
@@ -854,6 +861,9 @@ static void derive(cwc_model* m) {
     m->sumsq_d.resize(TS);
     const int nq = (int)m->quantiles.size();
     m->quant.assign(TS * nq, NAN);
+    std::vector<int> qorder(nq);
+    for (int qi = 0; qi < nq; ++qi) qorder[qi] = qi;
+    std::stable_sort(qorder.begin(), qorder.end(), [&](int a, int b) { return m->quantiles[a] < m->quantiles[b]; });
     for (int64_t k = 0; k < T; ++k) {
         m->times[k] = (double)k * m->dt;
         const int64_t n = m->h_n[k];
@@ -864,9 +874,8 @@ static void derive(cwc_model* m) {
             m->sumsq_d[i] = (double)sq;
             if (n > 0) m->mean[i] = (double)sum / (double)n;
             if (n > 1) m->var[i] = (double)((__int128)n * sq - sum * sum) / (double)((__int128)n * (n - 1));
-            for (int qi = 0; qi < nq; ++qi)
-                m->quant[i * nq + qi] = quantile_from_hist(&m->h_hist[i * (B + 2)], B, n, m->quantiles[qi],
-                                                           m->hist_lo[s], m->hist_width[s]);
+            quantiles_from_hist(&m->h_hist[i * (B + 2)], B, n, m->quantiles, qorder, m->hist_lo[s],
+                                m->hist_width[s], &m->quant[i * nq]);
         }
     }
     m->finalized = true;
