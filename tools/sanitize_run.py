@@ -48,6 +48,17 @@ def main():
     res = m.simulate(300, 3.0, 0.5, 5)
     assert res.finished == 300
     print("vesicles (dynamic pools) ok", flush=True)
+    # checkpoint / resume: terminate, save to host, restore into a fresh handle, resume
+    m = cwc.Model.from_def(W.SCHLOGL, hist_bins=64)
+    for cf, res in m.stream(4000, 1.0, 0.05, 11, poll_s=0.001, stop=lambda c, r: c > 0):
+        pass
+    ckpt = m.checkpoint()
+    m2 = cwc.Model.from_def(W.SCHLOGL, hist_bins=64)
+    m2.restore(ckpt)
+    m2.resume()
+    res = m2.finalize()
+    assert res.finished == 4000
+    print(f"checkpoint/resume ok (cuts final at stop {cf})", flush=True)
 
 
 if __name__ == "__main__":
