@@ -6,9 +6,12 @@
 
 One step = the whole hot path over one synthetic ensemble: instance
 generation, SSA to t_end, sampling on the grid, fused on-line statistics, and (N > 1) the
-NCCL all-reduce of the statistics.  Weak scaling: every rank simulates the configured number
-of instances (config "lv" = BASELINE.json configs[1]: Lotka-Volterra, 100k instances per GPU,
-t_end = 50, dt = 0.1), rank r owning global instances [r*n, (r+1)*n).
+NCCL all-reduce of the statistics.  Default workload: the north-star ensemble (BASELINE.json
+north_star, config "lv1m"): Lotka-Volterra, 1,000,000 instances, t_end = 50, dt = 0.1,
+STRONG scaling — the 1M instances are sharded over the N ranks (125k per GPU at N = 8), rank r
+owning the contiguous global range [floor(rN/G), floor((r+1)N/G)).  ``--scaling weak`` keeps
+the configured instances per GPU instead (e.g. ``--config lv --scaling weak``: BASELINE.json
+configs[1], 100k per GPU).
 
 Rank 0 prints ONE JSON line.  Timing: W warm-up steps, then K steps bracketed by barrier +
 synchronize; each step is timed with CUDA events on the launching stream after a 256 MiB L2
@@ -43,6 +46,18 @@ LOGTAB_BYTES = 3072  # CWC-log table uploaded once per model load (128 x {invc, 
 
 
 # ---------------------------------------------------------------------------------- helpers
+def measured_imin(model_name: str):
+    """I_min of SURVEY §8(d): thread-instructions per reaction of a divergence-free single-warp
+    run of this model's SSA kernel (tools/imin.py under ncu: smsp__inst_executed x 32 /
+    reactions), committed as profiles/imin_<model>.json for the kernel revision it measured."""
+    try:
+        with open(os.path.join(ROOT, "profiles", f"imin_{model_name}.json")) as f:
+            d = json.load(f)
+        return float(d["imin_thread_inst_per_reaction"]), d
+    except (OSError, KeyError, ValueError):
+        return None, None
+
+
 def algorithmic_instructions(info: dict) -> int:
     """Minimal thread-instruction count of one direct-method SSA step of this flat model on
     sm_100a (DESIGN.md §5 "algorithmic work"): the unit of the ALU roofline."""
@@ -169,7 +184,7 @@ def run_reference(args):
     line = {
         "impl": "reference", "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": args.gpus,
         "steps": args.steps, "warmup": args.warmup, "ms_per_step": 1e3 * tot_s / args.steps,
-        "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "f64", "data": "synthetic",
+        "higher_is_better": True, "scaling": args.scaling, "vs_baseline": None, "dtype": "f64", "data": "synthetic",
         "config": {"workload": args.config, "description": cfg.description},
         "trajectories_per_s": tot_i / tot_s,
         "cpu_baseline": {"value": value, "unit": UNIT, "cores": cores, "kind": "oracle",
@@ -193,12 +208,18 @@ def run_b200(args):
     rank = int(os.environ.get("RANK", "0"))
     local = int(os.environ.get("LOCAL_RANK", "0"))
     if world != args.gpus:
-        if world == 1 and args.gpus > 1:
-            print(f"--gpus {args.gpus} needs torchrun with {args.gpus} processes", file=sys.stderr)
-            return 2
-    # one process per GPU; CWC_DIST_BACKEND=gloo lets a functional multi-rank run share one GPU
+        print(f"--gpus {args.gpus} but WORLD_SIZE={world}: launch one process per GPU "
+              f"(torchrun --nproc-per-node {args.gpus})", file=sys.stderr)
+        return 2
+    # one process per GPU; CWC_DIST_BACKEND=gloo lets a functional multi-rank run share one GPU —
+    # such a line is tagged "shared_gpu" and is not a scaling point
     backend = os.environ.get("CWC_DIST_BACKEND", "nccl")
-    local = local % max(1, torch.cuda.device_count()) if backend != "nccl" else local
+    ndev = max(1, torch.cuda.device_count())
+    shared_gpu = world > ndev
+    if shared_gpu and backend == "nccl":
+        print(f"{world} ranks but {ndev} GPU(s): NCCL needs one GPU per rank", file=sys.stderr)
+        return 2
+    local = local % ndev
     torch.cuda.set_device(local)
     if world > 1:
         if backend == "nccl":
@@ -206,8 +227,11 @@ def run_b200(args):
         else:
             dist.init_process_group(backend)
     cfg = W.CONFIGS[args.config]
-    n_per = args.instances or cfg.n_instances
-    n_total = n_per * world
+    if args.scaling == "strong":
+        n_total = args.instances or cfg.n_instances
+    else:
+        n_total = (args.instances or cfg.n_instances) * world
+    n_per = n_total // world
 
     t0 = time.perf_counter()
     model = cwc.Model.from_def(cfg.model, hist_bins=cfg.hist_bins, hist_width=cfg.hist_width,
@@ -300,32 +324,42 @@ def run_b200(args):
         pass
     f_max = float(peaks.get("sm_max_mhz", 1965.0)) * 1e6
     i_alg = algorithmic_instructions(info)
+    i_min, imin_rec = measured_imin(cfg.model.name)
+    i_unit = i_min if i_min is not None else float(i_alg)
     reactions_per_launch = total_reactions / world
-    achieved = reactions_per_launch * i_alg / (kern_ms_max / 1e3) / 1e12
+    achieved = reactions_per_launch * i_unit / (kern_ms_max / 1e3) / 1e12
     peak = sms * 4 * 32 * f_max / 1e12
     raw_bytes = 0 if args.no_raw else res.n.size * len(info["names"]) * run.count * 4
-    traffic = None   # DRAM bytes per launch from the committed ncu --set full capture of this workload
-    try:
-        with open(os.path.join(ROOT, "profiles", f"traffic_{args.config}.json")) as f:
-            tr = json.load(f)
-        if world == 1 and not args.no_raw and run.count == W.CONFIGS[args.config].n_instances:
-            traffic = tr["dram_bytes_per_launch"]
-    except (OSError, KeyError, ValueError):
-        pass
+    traffic = None   # DRAM bytes per launch from a committed ncu --set full capture of this launch
+    import glob
+    for path in sorted(glob.glob(os.path.join(ROOT, "profiles", "traffic_*.json"))):
+        try:
+            with open(path) as f:
+                tr = json.load(f)
+            if (tr.get("workload") == args.config and int(tr.get("instances", -1)) == run.count
+                    and not args.no_raw):
+                traffic = tr["dram_bytes_per_launch"]
+        except (OSError, KeyError, ValueError):
+            continue
     roof = {"bound": "alu", "achieved": achieved, "peak": peak, "unit": "Tinst/s", "frac": achieved / peak,
             "traffic": traffic,
-            "detail": {"algorithmic_inst_per_reaction": i_alg, "sms": sms, "sm_clock_for_peak_mhz": f_max / 1e6,
+            "detail": {"unit": "I_min thread-instructions per reaction x reactions per launch / kernel time "
+                               "(SURVEY §8(d) useful fraction)" if i_min is not None else
+                               "I_alg (hand count; no measured I_min for this model)",
+                       "imin_thread_inst_per_reaction": i_min, "imin_source": (imin_rec or {}).get("source"),
+                       "algorithmic_inst_per_reaction": i_alg, "sms": sms, "sm_clock_for_peak_mhz": f_max / 1e6,
                        "peak_source": "148 SMs x 4 schedulers x 32 lanes x sm_max_mhz (MEASURED_PEAKS.json)",
                        "frac_at_measured_clock": (achieved / (sms * 128 * clk["sm_mhz"] * 1e6 / 1e12))
                        if clk.get("sm_mhz") else None,
                        "kernel_ms": kern_ms_max,
                        "algorithmic_bytes_per_launch": raw_bytes + run.buffers.stats.numel() * 8,
-                       "traffic_source": "profiles/traffic_<workload>.json (ncu --set full, dram read+write)",
+                       "traffic_source": "profiles/traffic_*.json of this workload and per-rank instance count "
+                                         "(ncu --set full, dram read+write of one launch)",
                        "sample_stream_gbs": (raw_bytes / (kern_ms_max / 1e3) / 1e9) if raw_bytes else 0.0}}
 
-    # ---- CPU baseline: the oracle on this host, rank 0 at N = 1 only
+    # ---- CPU baseline: the oracle on this host's cores, rank 0 (every N)
     cpu = None
-    if rank == 0 and world == 1 and not args.no_cpu_baseline:
+    if rank == 0 and not args.no_cpu_baseline:
         r_cpu, i_cpu, s_cpu, cores = oracle_sample(cfg, args.cpu_budget_s)
         cpu = {"value": r_cpu / s_cpu, "unit": UNIT, "cores": cores, "kind": "oracle",
                "sample": f"instances [0, {i_cpu}) of '{args.config}' at the full horizon, SSA + stats, "
@@ -334,12 +368,13 @@ def run_b200(args):
     if rank == 0:
         line = {
             "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": args.steps,
-            "warmup": args.warmup, "ms_per_step": ms_per_step, "higher_is_better": True, "scaling": "weak",
+            "warmup": args.warmup, "ms_per_step": ms_per_step, "higher_is_better": True, "scaling": args.scaling,
             "vs_baseline": None, "dtype": "f64", "data": "synthetic",
             "config": {"workload": args.config, "description": cfg.description, "instances_per_gpu": n_per,
                        "instances_total": n_total, "t_end": cfg.t_end, "sample_dt": cfg.sample_dt,
                        "cuts": int(res.n.size), "species": len(info["names"]), "flat_reactions": len(info["rates"]),
                        "raw_samples": not args.no_raw, "parallelism": f"dp{world} (instance sharding)",
+                       "shards": f"rank r simulates global instances [floor(r N/{world}), floor((r+1) N/{world}))",
                        "l2": "256 MiB buffer written before every timed step (outside the events)"},
             "trajectories_per_s": traj_s,
             "reactions_per_step": total_reactions,
@@ -358,6 +393,8 @@ def run_b200(args):
             "kernel": {**model.kernel_attributes(), "load_s": load_s},
             "stats_check": {"finished": res.finished, "absorbed": res.absorbed, "overflowed": res.overflowed},
         }
+        if shared_gpu:
+            line["shared_gpu"] = True   # functional multi-rank run on fewer GPUs: not a scaling point
         print(json.dumps(line), flush=True)
     if world > 1:
         dist.destroy_process_group()
@@ -369,9 +406,12 @@ def main(argv=None):
     ap.add_argument("--gpus", type=int, default=int(os.environ.get("WORLD_SIZE", "1")))
     ap.add_argument("--steps", type=int, default=5)
     ap.add_argument("--warmup", type=int, default=3)
-    ap.add_argument("--config", default="lv", choices=sorted(W.CONFIGS))
+    ap.add_argument("--config", default="lv1m", choices=sorted(W.CONFIGS))
+    ap.add_argument("--scaling", default="strong", choices=["strong", "weak"],
+                    help="strong: the config's instances split over the ranks; weak: that many per rank")
     ap.add_argument("--impl", default="b200", choices=["b200", "reference"])
-    ap.add_argument("--instances", type=int, default=0, help="instances per GPU (default: the config's)")
+    ap.add_argument("--instances", type=int, default=0,
+                    help="instances in total (strong) or per GPU (weak); default: the config's")
     ap.add_argument("--no-raw", action="store_true", help="do not keep raw samples (stats only)")
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--cpu-budget-s", type=float, default=15.0)

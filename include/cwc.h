@@ -364,6 +364,24 @@ cwc_status cwc_selftest_u01(int64_t n, const uint32_t* words, double* out); /* w
 /* The SSA kernel's branch-free IEEE division (round to nearest) for n pairs, host in/out. */
 cwc_status cwc_selftest_div(int64_t n, const double* num, const double* den, double* out);
 
+/* Injected-draw steps of a loaded model (test entry; SURVEY §8(c) "event forced onto a grid
+ * point (unit test with crafted u)").  The model's own NVRTC-compiled step code — mode 0: the
+ * SSA kernel's fast step followed by the full step when the lane leaves the fast path; mode 1:
+ * the full step only — runs n trajectories on the device, trajectory i starting from state
+ * x[i][S] at time t[i] with next cut index k[i] (0 <= k <= K+1, K = llround(t_end/sample_dt)),
+ * and takes up to n_draws steps with the uniforms u_tau[i][d], u_sel[i][d] in place of the
+ * Philox draws (R3), stopping after the first step that is not a jump.  The step is the
+ * direct method of P:L216-217 with the cut rule of P:L249-251 (reading R7) and the selection
+ * rule R6.  Outputs (host, caller-owned): x_out[i][S], t_out[i] (time of the last jump),
+ * k_out[i], status[i] = 0 jump / 2 horizon reached / 3 absorbed / 4 overflowed (the last step's),
+ * n_done[i] = steps taken, and (optional) cuts[i][K+1][S]: the cuts these steps emitted, -2 where
+ * none, -1 = missing after an overflow.  Errors: CWC_E_INVALID (bad sizes, k outside [0, K+1],
+ * mode not 0/1), CWC_E_CUDA (no device). */
+cwc_status cwc_selftest_step(cwc_model_t m, int64_t n, int32_t n_draws, const int32_t* x, const double* t,
+                             const int64_t* k, double t_end, double sample_dt, const double* u_tau,
+                             const double* u_sel, int32_t mode, int32_t* x_out, double* t_out, int64_t* k_out,
+                             int32_t* status, int32_t* n_done, int32_t* cuts);
+
 /* Library version string. */
 const char* cwc_version(void);
 

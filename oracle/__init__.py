@@ -92,6 +92,11 @@ def lib():
         _lib.oracle_simulate.restype = ctypes.c_int
         _lib.oracle_propensities.argtypes = [ctypes.POINTER(_Model), ctypes.c_void_p,
                                              ctypes.c_void_p, ctypes.c_void_p]
+        _lib.oracle_step_with_draws.argtypes = [
+            ctypes.POINTER(_Model), ctypes.c_void_p, ctypes.POINTER(ctypes.c_double), ctypes.POINTER(ctypes.c_int64),
+            ctypes.c_int64, ctypes.c_double, ctypes.c_int32, ctypes.c_void_p, ctypes.c_void_p, ctypes.c_void_p,
+            ctypes.c_void_p, ctypes.POINTER(ctypes.c_int32)]
+        _lib.oracle_step_with_draws.restype = ctypes.c_int
     return _lib
 
 
@@ -171,6 +176,43 @@ class CModel:
         cum = np.zeros(max(self.M, 1))
         lib().oracle_propensities(ctypes.byref(self.c), x.ctypes.data, a.ctypes.data, cum.ctypes.data)
         return a[: self.M], cum[: self.M]
+
+
+# status of an injected-draw step (ssa.c ssa_step)
+STEP_JUMP, STEP_ABSORBED, STEP_OVERFLOWED, STEP_HORIZON = 0, 1, 2, 3
+
+
+@dataclass
+class StepRun:
+    x: np.ndarray          # [S] state after the steps
+    t: float               # time of the last applied jump
+    k: int                 # next cut index
+    status: int            # STEP_* of the last step taken
+    n_done: int            # steps taken (the last one may be a non-jump)
+    js: np.ndarray         # [n_done] selected reaction of each step (-1: no jump)
+    cuts: np.ndarray       # [K+1][S] cuts emitted (-2 = not emitted by these steps, -1 = missing)
+
+
+def step_with_draws(model, x, t: float, k: int, K: int, dt: float, u_tau, u_sel) -> StepRun:
+    """Injected-draw trajectory: from state (x, t, next cut k), the direct-method steps of ssa.c
+    with the given uniforms instead of Philox draws (R6/R7 pins with crafted draws; the
+    device counterpart is cwc_selftest_step)."""
+    cm = model if isinstance(model, CModel) else CModel(model if isinstance(model, FlatModel) else flatten_def(model))
+    xs = np.ascontiguousarray(x, dtype=np.int32).copy()
+    ut = np.ascontiguousarray(u_tau, dtype=np.float64)
+    us = np.ascontiguousarray(u_sel, dtype=np.float64)
+    n = len(ut)
+    cuts = np.full((K + 1, cm.S), -2, dtype=np.int32)
+    js = np.full(max(n, 1), -1, dtype=np.int32)
+    tt = ctypes.c_double(t)
+    kk = ctypes.c_int64(k)
+    nd = ctypes.c_int32(0)
+    st = lib().oracle_step_with_draws(ctypes.byref(cm.c), xs.ctypes.data, ctypes.byref(tt), ctypes.byref(kk), K, dt,
+                                      n, ut.ctypes.data, us.ctypes.data, cuts.ctypes.data, js.ctypes.data,
+                                      ctypes.byref(nd))
+    if st < 0:
+        raise CWCError("invalid", "oracle_step_with_draws rejected its arguments")
+    return StepRun(xs, tt.value, kk.value, st, nd.value, js[: nd.value], cuts)
 
 
 def grid_K(t_end: float, dt: float) -> int:

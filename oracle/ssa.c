@@ -230,14 +230,81 @@ static void emit_missing(const job_t* jb, int64_t li, int64_t k) {
     for (int32_t s = 0; s < S; ++s) jb->raw[(k * S + s) * jb->count + li] = -1;
 }
 
-/* One instance, SURVEY.md §8(c) pseudo-code in order. */
-static void simulate_instance(const job_t* jb, int64_t li) {
+/* One direct-method step of instance li from state (x, *t, *k) with the draw (u_tau, u_sel),
+ * SURVEY.md §8(c) pseudo-code from "propensities" to "x += nu_{j*}", in that order:
+ *   ORACLE_STEP_ABSORBED   a0 == 0 (R8): cuts k..K hold x, the draw is not consumed
+ *   ORACLE_STEP_HORIZON    the next jump lies beyond t_K: cuts up to K emitted, no jump
+ *   ORACLE_STEP_OVERFLOWED the jump was applied and a count exceeds X_cap (R9): cuts k..K missing
+ *   ORACLE_STEP_JUMP       the jump was applied (cuts strictly before it emitted, R7)
+ * *js_out (optional) = the selected reaction j* (-1 when no jump was applied). */
+enum { ORACLE_STEP_JUMP = 0, ORACLE_STEP_ABSORBED = 1, ORACLE_STEP_OVERFLOWED = 2, ORACLE_STEP_HORIZON = 3 };
+
+static int ssa_step(const job_t* jb, int64_t li, int32_t* x, double* t, int64_t* k, double u_tau, double u_sel,
+                    int32_t* js_out) {
     const oracle_model* m = jb->m;
     const int32_t S = m->S, M = m->M;
     const int64_t K = jb->K;
+    static __thread double a[ORACLE_MMAX], cum[ORACLE_MMAX];
+    if (js_out) *js_out = -1;
+    /* propensities a_j = fl(k_j * (double)h_j), h_j = prod_s C(x_s, r_js) (R1) */
+    for (int32_t j = 0; j < M; ++j) {
+        uint64_t h = 1;
+        for (int32_t e = 0; e < m->n_react[j]; ++e)
+            h *= binom(x[m->react_s[j * ORACLE_RMAX + e]], m->react_r[j * ORACLE_RMAX + e]);
+        a[j] = propensity(m, j, x, h);
+    }
+    /* a0 as a left-to-right running sum (R5) */
+    double c = 0.0;
+    for (int32_t j = 0; j < M; ++j) { c = c + a[j]; cum[j] = c; }
+    double a0 = c;
+    if (a0 == 0.0) {                          /* absorbing state (R8): hold to t_K, no draw */
+        for (; *k <= K; ++*k) emit(jb, li, *k, x);
+        return ORACLE_STEP_ABSORBED;
+    }
+    double tau = -oracle_cwclog(u_tau) / a0;
+    double t_next = *t + tau;
+    /* cuts at t_k = fl(k*dt) strictly before the next jump: cadlag sampling (R7) */
+    while (*k <= K && (double)*k * jb->dt < t_next) { emit(jb, li, *k, x); ++*k; }
+    if (*k > K) return ORACLE_STEP_HORIZON;
+    /* rule selection (R6): j* = min{ j : cum_j > u_sel*a0 }, else last positive a_j */
+    double target = u_sel * a0;
+    int32_t js = -1;
+    for (int32_t j = 0; j < M; ++j) if (cum[j] > target) { js = j; break; }
+    if (js < 0) for (int32_t j = M - 1; j >= 0; --j) if (a[j] > 0.0) { js = j; break; }
+    if (js_out) *js_out = js;
+    /* multiset rewrite: x += nu_{j*} */
+    for (int32_t s = 0; s < S; ++s) x[s] += m->delta[js * S + s];
+    /* reading R20: a creation fills the first free slot of its pool; a destruction moves the
+     * rest of the dissolved compartment to the context (or removes it) */
+    if (m->place_off)
+        for (int32_t p = m->place_off[js]; p < m->place_off[js + 1]; ++p)
+            if (x[m->place_alive[p]] == 0) {
+                for (int32_t e = m->add_off[p]; e < m->add_off[p + 1]; ++e) x[m->add_s[e]] += m->add_n[e];
+                break;
+            }
+    if (m->xfer_off)
+        for (int32_t e = m->xfer_off[js]; e < m->xfer_off[js + 1]; ++e) {
+            if (m->xfer_dst[e] >= 0) x[m->xfer_dst[e]] += x[m->xfer_src[e]];
+            x[m->xfer_src[e]] = 0;
+        }
+    *t = t_next;
+    int over = 0;
+    for (int32_t s = 0; s < S; ++s) if (x[s] > m->x_cap) over = 1;
+    if (m->sentinel >= 0 && x[m->sentinel] > 0) over = 1;
+    if (over) {                               /* R9: freeze, remaining samples missing */
+        for (; *k <= K; ++*k) emit_missing(jb, li, *k);
+        return ORACLE_STEP_OVERFLOWED;
+    }
+    return ORACLE_STEP_JUMP;
+}
+
+/* One instance: the draw of step n is Philox4x32-10 block (ctr = (n, i), key = seed) (R3),
+ * mapped to two 52-bit uniforms; steps until absorption, overflow or the horizon. */
+static void simulate_instance(const job_t* jb, int64_t li) {
+    const oracle_model* m = jb->m;
+    const int32_t S = m->S;
     const uint64_t i = (uint64_t)(jb->first + li);
     int32_t x[ORACLE_SMAX];
-    static __thread double a[ORACLE_MMAX], cum[ORACLE_MMAX];
     for (int32_t s = 0; s < S; ++s) x[s] = m->x0[s];
     double t = 0.0;
     uint64_t step = 0;
@@ -245,66 +312,44 @@ static void simulate_instance(const job_t* jb, int64_t li) {
     uint8_t flag = 0;
     const uint32_t key[2] = {(uint32_t)jb->seed, (uint32_t)(jb->seed >> 32)};
     for (;;) {
-        /* propensities a_j = fl(k_j * (double)h_j), h_j = prod_s C(x_s, r_js) (R1) */
-        for (int32_t j = 0; j < M; ++j) {
-            uint64_t h = 1;
-            for (int32_t e = 0; e < m->n_react[j]; ++e)
-                h *= binom(x[m->react_s[j * ORACLE_RMAX + e]], m->react_r[j * ORACLE_RMAX + e]);
-            a[j] = propensity(m, j, x, h);
-        }
-        /* a0 as a left-to-right running sum (R5) */
-        double c = 0.0;
-        for (int32_t j = 0; j < M; ++j) { c = c + a[j]; cum[j] = c; }
-        double a0 = c;
-        if (a0 == 0.0) {                      /* absorbing state (R8): hold to t_K, no draw */
-            flag = ORACLE_FLAG_ABSORBED;
-            for (; k <= K; ++k) emit(jb, li, k, x);
-            break;
-        }
         uint32_t ctr[4] = {(uint32_t)step, (uint32_t)(step >> 32), (uint32_t)i, (uint32_t)(i >> 32)};
         uint32_t w[4];
         oracle_philox4x32_10(ctr, key, w);
         double u_tau = oracle_u01(w[0], w[1]);
         double u_sel = oracle_u01(w[2], w[3]);
-        double tau = -oracle_cwclog(u_tau) / a0;
-        double t_next = t + tau;
-        /* cuts at t_k = fl(k*dt) strictly before the next jump: cadlag sampling (R7) */
-        while (k <= K && (double)k * jb->dt < t_next) { emit(jb, li, k, x); ++k; }
-        if (k > K) break;
-        /* rule selection (R6): j* = min{ j : cum_j > u_sel*a0 }, else last positive a_j */
-        double target = u_sel * a0;
-        int32_t js = -1;
-        for (int32_t j = 0; j < M; ++j) if (cum[j] > target) { js = j; break; }
-        if (js < 0) for (int32_t j = M - 1; j >= 0; --j) if (a[j] > 0.0) { js = j; break; }
-        /* multiset rewrite: x += nu_{j*} */
-        for (int32_t s = 0; s < S; ++s) x[s] += m->delta[js * S + s];
-        /* reading R20: a creation fills the first free slot of its pool; a destruction moves the
-         * rest of the dissolved compartment to the context (or removes it) */
-        if (m->place_off)
-            for (int32_t p = m->place_off[js]; p < m->place_off[js + 1]; ++p)
-                if (x[m->place_alive[p]] == 0) {
-                    for (int32_t e = m->add_off[p]; e < m->add_off[p + 1]; ++e) x[m->add_s[e]] += m->add_n[e];
-                    break;
-                }
-        if (m->xfer_off)
-            for (int32_t e = m->xfer_off[js]; e < m->xfer_off[js + 1]; ++e) {
-                if (m->xfer_dst[e] >= 0) x[m->xfer_dst[e]] += x[m->xfer_src[e]];
-                x[m->xfer_src[e]] = 0;
-            }
-        t = t_next;
-        step += 1;
+        int st = ssa_step(jb, li, x, &t, &k, u_tau, u_sel, NULL);
+        if (st == ORACLE_STEP_ABSORBED) { flag = ORACLE_FLAG_ABSORBED; break; }
+        if (st == ORACLE_STEP_HORIZON) break;
+        step += 1;                            /* the draw was consumed: one reaction applied */
         reactions += 1;
-        int over = 0;
-        for (int32_t s = 0; s < S; ++s) if (x[s] > m->x_cap) over = 1;
-        if (m->sentinel >= 0 && x[m->sentinel] > 0) over = 1;
-        if (over) {                           /* R9: freeze, remaining samples missing */
-            flag = ORACLE_FLAG_OVERFLOWED;
-            for (; k <= K; ++k) emit_missing(jb, li, k);
-            break;
-        }
+        if (st == ORACLE_STEP_OVERFLOWED) { flag = ORACLE_FLAG_OVERFLOWED; break; }
     }
     if (jb->flags) jb->flags[li] = flag;
     if (jb->reactions) jb->reactions[li] = reactions;
+}
+
+/* Injected-draw trajectory (pins of R6/R7 with crafted uniforms; the device counterpart is
+ * cwc_selftest_step): from state (x, *t, *k), apply up to n_draws steps of ssa_step with the
+ * draws (u_tau[d], u_sel[d]), stopping at the first step that is not a jump.  Cuts emitted go to
+ * cuts[k][s] ([K+1][S], caller-initialised; -1 = missing after an overflow); js[d] (optional)
+ * receives the selected reactions.  Returns the status of the last step taken (ORACLE_STEP_*)
+ * and *n_done the number of steps taken (draws consumed + a final non-jump step). */
+int oracle_step_with_draws(const oracle_model* m, int32_t* x, double* t, int64_t* k, int64_t K, double dt,
+                           int32_t n_draws, const double* u_tau, const double* u_sel, int32_t* cuts, int32_t* js,
+                           int32_t* n_done) {
+    if (!m || m->S <= 0 || m->S > ORACLE_SMAX || m->M < 0 || m->M > ORACLE_MMAX || K < 0 || !(dt > 0) ||
+        n_draws < 0 || *k < 0 || *k > K + 1)
+        return -1;
+    pthread_once(&cwclog_once, cwclog_init);
+    job_t jb = {m, 0, 1, K, dt, 0, cuts, NULL, NULL, 0, 1};
+    int st = ORACLE_STEP_JUMP;
+    int32_t d = 0;
+    for (; d < n_draws; ++d) {
+        st = ssa_step(&jb, 0, x, t, k, u_tau[d], u_sel[d], js ? js + d : NULL);
+        if (st != ORACLE_STEP_JUMP) { ++d; break; }
+    }
+    if (n_done) *n_done = d;
+    return st;
 }
 
 static void* worker(void* arg) {

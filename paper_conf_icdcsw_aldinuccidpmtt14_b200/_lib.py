@@ -95,6 +95,8 @@ SIGNATURES = {
     "cwc_selftest_log": (c_i32, [c_i64, c_vp, c_vp]),
     "cwc_selftest_u01": (c_i32, [c_i64, c_vp, c_vp]),
     "cwc_selftest_div": (c_i32, [c_i64, c_vp, c_vp, c_vp]),
+    "cwc_selftest_step": (c_i32, [c_vp, c_i64, c_i32, c_vp, c_vp, c_vp, c_dbl, c_dbl, c_vp, c_vp, c_i32, c_vp, c_vp,
+                                  c_vp, c_vp, c_vp, c_vp]),
 }
 
 

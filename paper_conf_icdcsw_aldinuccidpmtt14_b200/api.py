@@ -352,6 +352,32 @@ class Model:
             return st.T
         raise CWCError(6, "finalize before reading samples")
 
+    def selftest_step(self, x, t, k, t_end: float, sample_dt: float, u_tau, u_sel, mode: int = 0) -> dict:
+        """Injected-draw steps on the device (cwc_selftest_step): trajectory i starts from
+        x[i], t[i], next cut k[i] and takes up to D steps with the uniforms u_tau[i][:D],
+        u_sel[i][:D].  mode 0 = the SSA kernel's fast step + full step, 1 = full step only."""
+        S = self.n_species
+        x = np.ascontiguousarray(x, dtype=np.int32).reshape(-1, S)
+        n = len(x)
+        t = np.ascontiguousarray(t, dtype=np.float64).reshape(n)
+        k = np.ascontiguousarray(k, dtype=np.int64).reshape(n)
+        ut = np.ascontiguousarray(u_tau, dtype=np.float64).reshape(n, -1)
+        us = np.ascontiguousarray(u_sel, dtype=np.float64).reshape(n, -1)
+        D = ut.shape[1]
+        if us.shape != ut.shape:
+            raise ValueError("u_tau and u_sel must have the same shape")
+        T = int(round(t_end / sample_dt)) + 1
+        xo = np.empty_like(x)
+        to = np.empty(n, dtype=np.float64)
+        ko = np.empty(n, dtype=np.int64)
+        st = np.empty(n, dtype=np.int32)
+        nd = np.empty(n, dtype=np.int32)
+        cuts = np.empty((n, T, S), dtype=np.int32)
+        check(lib.cwc_selftest_step(self._h, n, D, _ptr(x), _ptr(t), _ptr(k), float(t_end), float(sample_dt),
+                                    _ptr(ut), _ptr(us), int(mode), _ptr(xo), _ptr(to), _ptr(ko), _ptr(st), _ptr(nd),
+                                    _ptr(cuts)))
+        return {"x": xo, "t": to, "k": ko, "status": st, "n_done": nd, "cuts": cuts}
+
     def records(self, first: int, count: int):
         flags = np.empty(count, dtype=np.uint8)
         reactions = np.empty(count, dtype=np.int64)

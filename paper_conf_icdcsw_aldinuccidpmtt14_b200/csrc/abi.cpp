@@ -534,4 +534,17 @@ cwc_status cwc_selftest_u01(int64_t n, const uint32_t* w, double* out) {
     });
 }
 
+cwc_status cwc_selftest_step(cwc_model_t m, int64_t n, int32_t n_draws, const int32_t* x, const double* t,
+                             const int64_t* k, double t_end, double sample_dt, const double* u_tau,
+                             const double* u_sel, int32_t mode, int32_t* x_out, double* t_out, int64_t* k_out,
+                             int32_t* status, int32_t* n_done, int32_t* cuts) {
+    return guard([&] {
+        need(m != nullptr, "NULL model");
+        need(n >= 0 && (n == 0 || (x && t && k && u_tau && u_sel && x_out && t_out && k_out && status && n_done)),
+             "bad arguments");
+        cwc::selftest_step(m, n, n_draws, x, t, k, t_end, sample_dt, u_tau, u_sel, mode, x_out, t_out, k_out, status,
+                           n_done, cuts);
+    });
+}
+
 }  // extern "C"

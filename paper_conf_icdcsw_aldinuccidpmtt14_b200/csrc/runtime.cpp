@@ -655,6 +655,9 @@ void cancel(cwc_model* m) {
     if (!m->poll_stream) ck(cudaStreamCreateWithFlags(&m->poll_stream, cudaStreamNonBlocking), "cudaStreamCreate");
     static const uint32_t one = 1;
     const ScratchLayout L = scratch_layout(m->fm.S(), m->count, m->K + 1);
+    // the flag lives in the range simulate_range clears on the launch stream before ev0: order the
+    // write after that memset, or a cancel issued while it is still queued would be erased
+    ck(cudaStreamWaitEvent(m->poll_stream, m->ev0, 0), "order cancel after the launch's memsets");
     ck(cudaMemcpyAsync((char*)m->d_scratch + L.cancel, &one, 4, cudaMemcpyHostToDevice, m->poll_stream),
        "set cancel flag");
     ck(cudaStreamSynchronize(m->poll_stream), "set cancel flag");
@@ -753,6 +756,19 @@ void checkpoint_load(cwc_model* m, const void* in, size_t bytes) {
     std::memcpy(&h, in, sizeof h);
     if (std::memcmp(h.magic, kCkptMagic, 8) != 0) fail(CWC_E_INVALID, "not a checkpoint");
     if (h.identity != model_identity(m)) fail(CWC_E_INVALID, "checkpoint of a different model or options");
+    // the header sizes every buffer and the work-item geometry: validate it before any use
+    if (!(h.dt > 0) || !std::isfinite(h.dt) || !(h.t_end >= 0) || !std::isfinite(h.t_end))
+        fail(CWC_E_INVALID, "checkpoint header: bad horizon or sample interval");
+    int64_t K_hdr = -1;
+    try {
+        K_hdr = grid_K(h.t_end, h.dt);
+    } catch (const Error&) {
+        fail(CWC_E_INVALID, "checkpoint header: t_end is not a multiple of sample_dt");
+    }
+    if (h.K != K_hdr) fail(CWC_E_INVALID, "checkpoint header: K does not match t_end / sample_dt");
+    if (h.qs < 1 || h.qs > h.K + 1) fail(CWC_E_INVALID, "checkpoint header: quantum outside [1, K+1]");
+    if (h.n_total <= 0 || h.first < 0 || h.count < 0 || h.first > h.n_total || h.count > h.n_total - h.first)
+        fail(CWC_E_INVALID, "checkpoint header: instance range outside [0, n_total)");
     size_t ns, nr, nsc;
     buffer_sizes(m, h.count, h.K, &ns, &nr, &nsc);
     if (ns != h.stats_len || nr != h.raw_len || nsc != h.scratch_bytes ||
@@ -919,6 +935,112 @@ void copy_records(cwc_model* m, int64_t first, int64_t count, uint8_t* flags, in
     if (reactions)
         ck(cudaMemcpy(reactions, sc + L.step + first * 8, count * 8, cudaMemcpyDeviceToHost), "copy reactions");
     if (t_last) ck(cudaMemcpy(t_last, sc + L.t + first * 8, count * 8, cudaMemcpyDeviceToHost), "copy times");
+}
+
+
+// ------------------------------------------------------------------------ injected-draw self-test
+// The SSA kernel's own step code (cwc_step_selftest_kernel in cwc_ssa.cuh, same NVRTC module)
+// driven by caller-supplied uniforms from caller-supplied states: one lane per trajectory, up to
+// n_draws steps each.  Host arrays in and out; cuts[i][k][s] = -2 where this call emitted no cut.
+namespace {
+struct SelftestIo {  // mirrors cwc_selftest_io (cwc_ssa.cuh)
+    const int* x_in;
+    const double* t_in;
+    const long long* k_in;
+    const double* u_tau;
+    const double* u_sel;
+    int* x_out;
+    double* t_out;
+    long long* k_out;
+    int* status;
+    int* n_done;
+    long long n;
+    int D;
+    int mode;
+};
+}  // namespace
+
+void selftest_step(cwc_model* m, int64_t n, int32_t n_draws, const int32_t* x, const double* t, const int64_t* k,
+                   double t_end, double dt, const double* u_tau, const double* u_sel, int32_t mode, int32_t* x_out,
+                   double* t_out, int64_t* k_out, int32_t* status, int32_t* n_done, int32_t* cuts) {
+    if (n < 0 || n_draws < 1 || (mode != 0 && mode != 1)) fail(CWC_E_INVALID, "bad self-test arguments");
+    const int64_t K = grid_K(t_end, dt), T = K + 1;
+    const int S = m->fm.S();
+    for (int64_t i = 0; i < n; ++i)
+        if (k[i] < 0 || k[i] > T) fail(CWC_E_INVALID, "next cut index outside [0, K+1]");
+    if (n == 0) return;
+    compile(m, nullptr);
+    const int dev = current_device(m);
+    ensure_module(m, dev);
+    Driver& d = driver();
+    CUfunction fn = nullptr;
+    ckd(d.ModuleGetFunction(&fn, m->module, "cwc_step_selftest_kernel"), "cuModuleGetFunction(selftest)");
+    cwc_logtab_entry tab[128];
+    build_log_table(tab);
+    const size_t TB = (size_t)((T + CWC_RAW_BLOCK - 1) / CWC_RAW_BLOCK);
+    const size_t raw_n = TB * S * (size_t)n * CWC_RAW_BLOCK;
+    const size_t st_n = stats_len(T, S, m->hist_bins, m->period_species >= 0);
+    const size_t nd = (size_t)n * n_draws;
+    // one device block: [logtab | stats | raw | x_in | t | k | u_tau | u_sel | x_out | t_out | k_out | status | n_done]
+    size_t off[14], o = 0;
+    const size_t sizes[13] = {sizeof tab, st_n * 8, raw_n * 4, (size_t)n * S * 4, (size_t)n * 8, (size_t)n * 8,
+                              nd * 8, nd * 8, (size_t)n * S * 4, (size_t)n * 8, (size_t)n * 8, (size_t)n * 4,
+                              (size_t)n * 4};
+    for (int i = 0; i < 13; ++i) { off[i] = o; o = align256(o + sizes[i]); }
+    off[13] = o;
+    char* dmem = nullptr;
+    ck(cudaMalloc(&dmem, o), "cudaMalloc(self-test)");
+    struct Free { char* p; ~Free() { cudaFree(p); } } guard_mem{dmem};
+    std::vector<int32_t> raw_init(raw_n, -2);
+    std::vector<long long> kk(k, k + n);
+    ck(cudaMemcpy(dmem + off[0], tab, sizeof tab, cudaMemcpyHostToDevice), "H2D");
+    ck(cudaMemset(dmem + off[1], 0, st_n * 8), "memset");
+    ck(cudaMemcpy(dmem + off[2], raw_init.data(), raw_n * 4, cudaMemcpyHostToDevice), "H2D");
+    ck(cudaMemcpy(dmem + off[3], x, (size_t)n * S * 4, cudaMemcpyHostToDevice), "H2D");
+    ck(cudaMemcpy(dmem + off[4], t, (size_t)n * 8, cudaMemcpyHostToDevice), "H2D");
+    ck(cudaMemcpy(dmem + off[5], kk.data(), (size_t)n * 8, cudaMemcpyHostToDevice), "H2D");
+    ck(cudaMemcpy(dmem + off[6], u_tau, nd * 8, cudaMemcpyHostToDevice), "H2D");
+    ck(cudaMemcpy(dmem + off[7], u_sel, nd * 8, cudaMemcpyHostToDevice), "H2D");
+    cwc_params P;
+    std::memset(&P, 0, sizeof P);
+    P.first = 0;
+    P.count = n;
+    P.K = K;
+    P.dt = dt;
+    P.qs = T;
+    P.n_items = n;
+    for (int r = 0; r < 10; ++r) {  // seed 0 (the primed Philox draws are overwritten by the injected ones)
+        P.rk.k0[r] = (uint32_t)r * 0x9E3779B9u;
+        P.rk.k1[r] = (uint32_t)r * 0xBB67AE85u;
+    }
+    P.stats = (unsigned long long*)(dmem + off[1]);
+    P.raw = (int*)(dmem + off[2]);
+    P.logtab = (const cwc_logtab_entry*)(dmem + off[0]);
+    P.smem_stats = 0;
+    SelftestIo io{(const int*)(dmem + off[3]), (const double*)(dmem + off[4]), (const long long*)(dmem + off[5]),
+                  (const double*)(dmem + off[6]), (const double*)(dmem + off[7]), (int*)(dmem + off[8]),
+                  (double*)(dmem + off[9]), (long long*)(dmem + off[10]), (int*)(dmem + off[11]),
+                  (int*)(dmem + off[12]), (long long)n, n_draws, mode};
+    void* args[] = {&P, &io};
+    const unsigned block = 128;
+    ckd(d.LaunchKernel(fn, (unsigned)((n + block - 1) / block), 1, 1, block, 1, 1, 0, nullptr, args, nullptr),
+        "cuLaunchKernel(self-test)");
+    ck(cudaDeviceSynchronize(), "self-test kernel");
+    std::vector<int32_t> raw(raw_n);
+    std::vector<long long> ko(n);
+    ck(cudaMemcpy(raw.data(), dmem + off[2], raw_n * 4, cudaMemcpyDeviceToHost), "D2H");
+    ck(cudaMemcpy(x_out, dmem + off[8], (size_t)n * S * 4, cudaMemcpyDeviceToHost), "D2H");
+    ck(cudaMemcpy(t_out, dmem + off[9], (size_t)n * 8, cudaMemcpyDeviceToHost), "D2H");
+    ck(cudaMemcpy(ko.data(), dmem + off[10], (size_t)n * 8, cudaMemcpyDeviceToHost), "D2H");
+    ck(cudaMemcpy(status, dmem + off[11], (size_t)n * 4, cudaMemcpyDeviceToHost), "D2H");
+    ck(cudaMemcpy(n_done, dmem + off[12], (size_t)n * 4, cudaMemcpyDeviceToHost), "D2H");
+    for (int64_t i = 0; i < n; ++i) k_out[i] = ko[i];
+    if (cuts)  // time-blocked [TB][S][n][8] -> [n][T][S]
+        for (int64_t i = 0; i < n; ++i)
+            for (int64_t kc = 0; kc < T; ++kc)
+                for (int s = 0; s < S; ++s)
+                    cuts[(i * T + kc) * S + s] =
+                        raw[(((size_t)(kc / CWC_RAW_BLOCK) * S + s) * n + i) * CWC_RAW_BLOCK + kc % CWC_RAW_BLOCK];
 }
 
 }  // namespace cwc

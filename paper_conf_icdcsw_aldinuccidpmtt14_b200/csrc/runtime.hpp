@@ -127,5 +127,8 @@ void selftest_log(int64_t n, const double* x, double* out);
 void selftest_u01(int64_t n, const uint32_t* words, double* out);
 void selftest_div(int64_t n, const double* num, const double* den, double* out);
 void build_log_table(cwc_logtab_entry* tab);
+void selftest_step(cwc_model* m, int64_t n, int32_t n_draws, const int32_t* x, const double* t, const int64_t* k,
+                   double t_end, double dt, const double* u_tau, const double* u_sel, int32_t mode, int32_t* x_out,
+                   double* t_out, int64_t* k_out, int32_t* status, int32_t* n_done, int32_t* cuts);
 
 }  // namespace cwc

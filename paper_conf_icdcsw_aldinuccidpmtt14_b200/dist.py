@@ -67,20 +67,42 @@ def simulate_sharded(model, n_total: int, t_end: float, sample_dt: float, seed: 
     return run.result()
 
 
+_HOST_GROUPS = {}
+
+
+def host_group(group=None):
+    """A CPU (gloo) process group over the ranks of ``group`` for host-resident buffers.
+
+    Snapshots are host numpy arrays taken while each rank's SSA kernel still occupies its GPU:
+    reducing them through NCCL would queue the collective behind that persistent kernel (and NCCL
+    kernels cannot get SMs while it runs), so the on-line combine would only complete when the
+    shard's whole simulation has ended.  A gloo group keeps them on the host.  Created once per
+    group; collective on first use (every rank of the world calls combine_partial together)."""
+    import torch.distributed as dist
+    if dist.get_backend(group) == "gloo":
+        return group
+    key = None if group is None else tuple(dist.get_process_group_ranks(group))
+    if key not in _HOST_GROUPS:
+        _HOST_GROUPS[key] = dist.new_group(ranks=None if key is None else list(key), backend="gloo")
+    return _HOST_GROUPS[key]
+
+
 def combine_partial(packed, cuts_final: int, group=None):
     """SUM the packed statistics and MIN the final-cut prefixes across ranks (host numpy in,
-    host numpy out): the combination rule of on-line multi-GPU streaming."""
+    host numpy out): the combination rule of on-line multi-GPU streaming.  The reduction runs on
+    a CPU (gloo) group (``host_group``): it never touches the device, so it completes while the
+    ranks' kernels are still running."""
     import numpy as np
     import torch
     import torch.distributed as dist
     buf = torch.from_numpy(np.ascontiguousarray(packed, dtype=np.int64).copy())
     cf = torch.tensor([int(cuts_final)], dtype=torch.int64)
-    if dist.is_available() and dist.is_initialized() and dist.get_world_size(group) > 1:
-        if dist.get_backend(group) == "nccl":
-            buf, cf = buf.cuda(), cf.cuda()
-        dist.all_reduce(buf, op=dist.ReduceOp.SUM, group=group)
-        dist.all_reduce(cf, op=dist.ReduceOp.MIN, group=group)
-    return buf.cpu().numpy(), int(cf.cpu()[0])
+    if dist.is_available() and dist.is_initialized():
+        hg = host_group(group)
+        if dist.get_world_size(hg) > 1:
+            dist.all_reduce(buf, op=dist.ReduceOp.SUM, group=hg)
+            dist.all_reduce(cf, op=dist.ReduceOp.MIN, group=hg)
+    return buf.numpy(), int(cf[0])
 
 
 def snapshot_sharded(model, group=None):

@@ -8,14 +8,15 @@ from oracle.stats import ensemble_stats
 
 
 def gpu_run(model_def, n_total, first, count, t_end, dt, seed, *, hist_bins=256, hist_width=1, hist_lo=0,
-            quantiles=(0.05, 0.25, 0.5, 0.75, 0.95), raw=True, **opts):
-    """Product path: load, simulate [first, first+count), return (result, raw, flags, reactions, model)."""
+            quantiles=(0.05, 0.25, 0.5, 0.75, 0.95), raw=True, copy_raw=True, **opts):
+    """Product path: load, simulate [first, first+count), return (result, raw, flags, reactions, model)
+    (raw = None when raw samples are off or copy_raw is False; read them with model.samples)."""
     import paper_conf_icdcsw_aldinuccidpmtt14_b200 as cwc
     m = cwc.Model.from_def(model_def, hist_bins=hist_bins, hist_width=hist_width, hist_lo=hist_lo,
                            quantiles=quantiles, raw_samples=raw, **opts)
     m.simulate_range(n_total, first, count, t_end, dt, seed)
     res = m.finalize()
-    samples = m.samples(0, count) if raw else None
+    samples = m.samples(0, count) if raw and copy_raw else None
     flags, reactions, _ = m.records(0, count)
     return res, samples, flags, reactions, m
 

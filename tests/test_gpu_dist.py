@@ -1,7 +1,7 @@
 """GPU: the multi-rank path end to end (torchrun, ranks sharing the available GPU(s)).
 
-Rank shards + all-reduce of the packed statistics must equal one run of the whole ensemble
-(DESIGN.md §6).  Uses NCCL when there is one GPU per rank, gloo otherwise (one B200 here).
+Rank shards + all-reduce of the packed statistics must equal the oracle's statistics of the
+whole ensemble and one GPU run of it.  Uses NCCL when there is one GPU per rank, gloo otherwise (one B200 here).
 """
 import os
 import socket
@@ -30,7 +30,7 @@ def test_torchrun_sharded_equals_whole(nproc):
     if torch.cuda.device_count() < nproc:
         env["CWC_DIST_BACKEND"] = "gloo"
     cmd = [sys.executable, "-m", "torch.distributed.run", "--nnodes=1", f"--nproc-per-node={nproc}",
-           "--master-addr", "127.0.0.1", "--master-port", str(_port()), os.path.join(ROOT, "tools", "dist_check.py")]
+           "--master-addr", "127.0.0.1", "--master-port", str(_port()), os.path.join(ROOT, "tests", "workers", "dist_check.py")]
     r = subprocess.run(cmd, env=env, capture_output=True, text=True, timeout=600)
     assert r.returncode == 0, r.stdout[-3000:] + r.stderr[-3000:]
     assert "DIST OK" in r.stdout, r.stdout[-3000:]

@@ -124,3 +124,31 @@ def test_hill_autorepressor_stationary_1m():
     m, v, mu4 = _pmf_moments(xs.astype(np.float64), pi)
     for kk in (3, 4):                          # t = 15, 20: 15+ relaxation times from x0 = 0
         _check_mean_var(res.mean[kk, 0], res.var[kk, 0], N, m, v, mu4, f"t={res.times[kk]}")
+
+
+def _birth_death_pi(lam, mu, xmax=600):
+    """pi(x+1) / pi(x) = lam(x) / mu(x+1) (detailed balance of a birth-death chain)."""
+    xs = np.arange(xmax)
+    logpi = np.zeros(xs.size)
+    for x in range(1, xs.size):
+        logpi[x] = logpi[x - 1] + math.log(lam(x - 1) / mu(x))
+    pi = np.exp(logpi - logpi.max())
+    return xs.astype(np.float64), pi / pi.sum()
+
+
+@pytest.mark.parametrize("name", ["hill_act", "mm_death"])
+def test_functional_law_stationary_1m(name):
+    """Hill-ACTIVATED birth and Michaelis-Menten death (R16') at 1M instances: the finalised mean
+    and variance of the fused statistics within 4 SE of the detailed-balance stationary law."""
+    md = W.TINY_MODELS[name]
+    if name == "hill_act":
+        k0, k, mu = md.rates
+        xs, pi = _birth_death_pi(lambda x: k0 + k * x ** 2 / (15.0 ** 2 + x ** 2), lambda x: mu * x)
+    else:
+        k0, V = md.rates
+        xs, pi = _birth_death_pi(lambda x: k0, lambda x: V * x / (10.0 + x))
+    N = 1_000_000
+    res, *_ = gpu_run(md, N, 0, N, 40.0, 10.0, 91, hist_bins=512, raw=False)
+    m, v, mu4 = _pmf_moments(xs, pi)
+    for kk in (3, 4):                          # t = 30, 40: far past the relaxation time
+        _check_mean_var(res.mean[kk, 0], res.var[kk, 0], N, m, v, mu4, f"{name} t={res.times[kk]}")

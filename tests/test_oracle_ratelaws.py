@@ -32,18 +32,21 @@ def test_law_propensities_formulas():
         assert a[3] == ((1.5 * B) / (2.0 + B) if x[2] else 0.0)
 
 
-def test_autorepressor_stationary_law():
-    from scipy.stats import chi2
-    m = W.AUTOREPRESSOR
-    k, mu = m.rates
-    K, n = 30.0, 2
-    xs = np.arange(0, 200)
-    lam = k * K ** n / (K ** n + xs.astype(float) ** n)
-    logp = np.concatenate([[0.0], np.cumsum(np.log(lam[:-1]) - np.log(mu * xs[1:]))])
+def birth_death_law(lam, mu, xmax=400):
+    """Stationary law of a birth-death chain with birth rate lam(x) and death rate mu(x) (x >= 1):
+    detailed balance pi(x+1) mu(x+1) = pi(x) lam(x), i.e. pi(x) ∝ prod_{y<x} lam(y) / mu(y+1)."""
+    xs = np.arange(0, xmax)
+    lam_v = np.array([lam(float(y)) for y in xs])
+    mu_v = np.array([mu(float(y)) for y in xs[1:]])
+    logp = np.concatenate([[0.0], np.cumsum(np.log(lam_v[:-1]) - np.log(mu_v))])
     p = np.exp(logp - logp.max())
-    p /= p.sum()
-    N = 20000
-    run = oracle.simulate(flatten_def(m), 0, N, 12.0, 12.0, seed=8, nthreads=8)   # t = 12/mu: mixed
+    return xs, p / p.sum()
+
+
+def _fits_law(md, lam, mu, t_mix, seed, N=20000):
+    from scipy.stats import chi2
+    xs, p = birth_death_law(lam, mu)
+    run = oracle.simulate(flatten_def(md), 0, N, t_mix, t_mix, seed=seed, nthreads=8)   # one cut at t_mix
     x = run.raw[-1, 0]
     obs = np.bincount(x, minlength=len(p))[: len(p)].astype(float)
     exp = p * N
@@ -53,6 +56,31 @@ def test_autorepressor_stationary_law():
     mean = float((xs * p).sum())
     var = float(((xs - mean) ** 2 * p).sum())
     assert abs(x.mean() - mean) <= 4 * math.sqrt(var / N)
+    return mean
+
+
+def test_autorepressor_stationary_law():
+    """Hill-REPRESSED birth lambda(x) = k K^n / (K^n + x^n), linear death (law hillr)."""
+    k, mu = W.AUTOREPRESSOR.rates
+    K, n = 30.0, 2
+    _fits_law(W.AUTOREPRESSOR, lambda x: k * K ** n / (K ** n + x ** n), lambda x: mu * x, 12.0, 8)
+
+
+def test_hill_activated_birth_stationary_law():
+    """Hill-ACTIVATED birth lambda(x) = k0 + k x^n / (K^n + x^n) (law hill, R16'), linear death.
+    A dropped basal term, a swapped K^n / x^n or a wrong exponent moves the law far outside."""
+    k0, k, mu = W.HILL_ACT.rates
+    K, n = 15.0, 2
+    mean = _fits_law(W.HILL_ACT, lambda x: k0 + k * x ** n / (K ** n + x ** n), lambda x: mu * x, 15.0, 21)
+    assert 30.0 < mean < 40.0     # the positive feedback lifts the mean well above the basal 10
+
+
+def test_michaelis_menten_death_stationary_law():
+    """Constant birth k0, Michaelis-Menten death mu(x) = V x / (Km + x) (law mm, R16')."""
+    k0, V = W.MM_DEATH.rates
+    Km = 10.0
+    mean = _fits_law(W.MM_DEATH, lambda x: k0, lambda x: V * x / (Km + x), 30.0, 22)
+    assert 15.0 < mean < 40.0
 
 
 def test_neurospora_oscillates_with_published_period():

@@ -1,11 +1,13 @@
-"""Multi-rank functional check of the sharded path (dist.simulate_sharded) on the GPU box.
+"""Worker of tests/test_gpu_dist.py: multi-rank check of the sharded path (dist.simulate_sharded).
 
-    torchrun --nnodes=1 --nproc-per-node 2 --master-addr 127.0.0.1 --master-port 29511 tools/dist_check.py
+    torchrun --nnodes=1 --nproc-per-node 2 --master-addr 127.0.0.1 --master-port 29511 tests/workers/dist_check.py
 
 With CWC_DIST_BACKEND=gloo every rank may share one GPU (functional test of the multi-rank
 code path when only one GPU is available); with the default nccl each rank needs its own GPU.
-Rank 0 compares the all-reduced statistics with a single-process run of the whole ensemble
-and prints "DIST OK" (exit code 1 on a mismatch).
+Rank 0 compares the all-reduced statistics with the ORACLE's statistics of the
+whole ensemble (oracle.simulate + oracle.stats.ensemble_stats: integers n / sum / sumsq / hist
+exact, mean / variance / quantiles bit-identical) and with a single-process GPU run, and prints
+"DIST OK" (exit code 1 on a mismatch).
 """
 import os
 import sys
@@ -17,7 +19,9 @@ import torch.distributed as dist
 ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 sys.path.insert(0, ROOT)
 
+import oracle  # noqa: E402
 import workloads as W  # noqa: E402
+from oracle.stats import ensemble_stats  # noqa: E402
 import paper_conf_icdcsw_aldinuccidpmtt14_b200 as cwc  # noqa: E402
 from paper_conf_icdcsw_aldinuccidpmtt14_b200.dist import simulate_sharded  # noqa: E402
 
@@ -34,14 +38,29 @@ def main():
         dist.init_process_group(backend)
     rank, world = dist.get_rank(), dist.get_world_size()
     md, N, t_end, dt, seed = W.SCHLOGL, 20011, 2.0, 0.1, 99
-    m = cwc.Model.from_def(md, hist_bins=512, device=local)
+    qs = (0.05, 0.25, 0.5, 0.75, 0.95)
+    m = cwc.Model.from_def(md, hist_bins=512, device=local, quantiles=qs)
     res = simulate_sharded(m, N, t_end, dt, seed)
     ok = True
     if rank == 0:
-        ref = cwc.Model.from_def(md, hist_bins=512, device=local).simulate(N, t_end, dt, seed)
+        ref = cwc.Model.from_def(md, hist_bins=512, device=local, quantiles=qs).simulate(N, t_end, dt, seed)
         for name in ("n", "sum", "sqlo", "sqhi", "hist"):
             ok &= bool(np.array_equal(getattr(res, name), getattr(ref, name)))
         ok &= res.reactions == ref.reactions and res.finished == N
+        # the combined statistics against the oracle's statistics of the whole ensemble
+        orun = oracle.simulate(md, 0, N, t_end, dt, seed, nthreads=os.cpu_count() or 1)
+        st = ensemble_stats(orun.raw, [0], [1], 512, qs)
+        exact = res.sumsq_exact()
+        ok_oracle = bool(np.array_equal(res.n, st.n) and np.array_equal(res.hist, st.hist))
+        ok_oracle &= all(int(res.sum[k, 0]) == st.sum[k, 0] and exact[k, 0] == st.sumsq[k, 0]
+                         for k in range(res.n.size))
+        ok_oracle &= bool(np.array_equal(res.mean, st.mean, equal_nan=True) and
+                          np.array_equal(res.var, st.var, equal_nan=True) and
+                          np.array_equal(res.quantile, st.quantile, equal_nan=True))
+        ok_oracle &= res.reactions == int(orun.reactions.sum())
+        print(f"oracle comparison of the all-reduced statistics: {'equal' if ok_oracle else 'DIFFERENT'}",
+              flush=True)
+        ok &= ok_oracle
     # on-line streaming across ranks (dist.snapshot_sharded): combined partial results while the
     # shards run; the final-cut prefix of every combined snapshot equals the whole run's
     import time

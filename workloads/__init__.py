@@ -141,6 +141,10 @@ CONFIGS: Dict[str, RunConfig] = {
                            description="immigration-death, 1,000 instances, t_end=100, dt=1"),
     "lv": RunConfig(2, LOTKA_VOLTERRA, 100_000, 50.0, 0.1, SEED_BASE + 2, 1024, 128,
                     description="Lotka-Volterra, 100k instances, t_end=50, dt=0.1"),
+    # the north-star run (BASELINE.json north_star: "a 1M-instance Lotka-Volterra ensemble"): the
+    # bench headline, strong-scaled over 1/2/4/8 GPUs (125k instances per GPU at 8)
+    "lv1m": RunConfig(2, LOTKA_VOLTERRA, 1_000_000, 50.0, 0.1, SEED_BASE + 2, 1024, 128,
+                      description="Lotka-Volterra, 1M instances (north-star ensemble), t_end=50, dt=0.1"),
     "schlogl": RunConfig(3, SCHLOGL, 1_000_000, 50.0, 0.1, SEED_BASE + 3, 1024, 1,
                          description="Schlogl bistable, 1M instances, t_end=50, dt=0.1"),
     "circadian": RunConfig(4, CIRCADIAN, 10_000_000, 48.0, 0.5, SEED_BASE + 4, 1024, 4,
@@ -211,6 +215,14 @@ PERIOD_ANALYSIS = {"neurospora": dict(species="M", lo=100, hi=350, window=48),
 AUTOREPRESSOR = ModelDef("autorepressor", ("P",), ("top: . -> P @ hillr(P, 30, 2)", "top: P -> ."),
                          (60.0, 1.0), ".")
 TINY_MODELS[AUTOREPRESSOR.name] = AUTOREPRESSOR
+# Hill-ACTIVATED birth (positive feedback, unimodal: lambda'(x*) ~ 0.22 < 1) on top of a basal birth,
+# linear death; and constant birth with Michaelis-Menten death.  Both are birth-death chains
+# whose stationary laws follow from detailed balance (tests/test_oracle_ratelaws.py)
+HILL_ACT = ModelDef("hill_act", ("P",), ("top: . -> P", "top: . -> P @ hill(P, 15, 2)", "top: P -> ."),
+                    (10.0, 30.0, 1.0), ".")
+MM_DEATH = ModelDef("mm_death", ("P",), ("top: . -> P", "top: P -> . @ mm(P, 10)"), (20.0, 30.0), ".")
+TINY_MODELS[HILL_ACT.name] = HILL_ACT
+TINY_MODELS[MM_DEATH.name] = MM_DEATH
 
 # --- dynamic compartments (reading R20, bounded pools) ------------------------
 # Vesicle traffic shaped like the paper's compartment creation/destruction: a
