@@ -204,7 +204,13 @@ cwc_status cwc_bind_device_buffers(cwc_model_t m, int64_t* stats, size_t stats_l
                                    size_t raw_len, void* scratch, size_t scratch_bytes);
 
 /* ------------------------------------------------------------------------------------------
- * Simulation — the hot path.
+ * Simulation — the hot path.  PAPER.md: "Monte Carlo methods applied to a number of independent
+ * instances ... an embarrassingly parallel problem: ... groups of instances can be executed
+ * independently" (§I); each instance is a trajectory of "the Gillespie algorithm on CWC
+ * terms" (§IV); trajectories are cut "at a given simulation time" and the
+ * cuts analysed on line (§IV.A.1-2); simulation quanta with re-scheduling (P:L241-243,
+ * §IV.A.1; GPU variant P:L300-317, §IV.C); one ff_mapCUDA per GPU = one shard per device
+ * (P:L304-305).  Readings R1-R15 fix what the paper leaves open.
  * cwc_simulate_range simulates the global instances [first, first+count) of an ensemble of
  * n_total instances, from t = 0 to t_end, sampling at t_k = fl(k*sample_dt), k = 0..K,
  * K = llround(t_end/sample_dt) (R7, R13).  Instance i uses the Philox stream keyed by
@@ -224,19 +230,28 @@ cwc_status cwc_simulate(cwc_model_t m, int64_t n_instances, double t_end, double
 cwc_status cwc_simulate_range(cwc_model_t m, int64_t n_total, int64_t first, int64_t count,
                               double t_end, double sample_dt, uint64_t seed, void* cuda_stream);
 
-/* Packed int64 statistics buffer, T = K+1 cuts, S species, B bins (all exact integers,
+/* Packed int64 statistics buffer — the per-cut "statistical estimators (mean, variance ...)"
+ * of the analysis pipeline (Fig. 2; on-line estimators P:L689-691; every cut "can be
+ * analysed immediately and independently" P:L249-251) and the cut histograms of GPU ensemble
+ * tools, accumulated exactly inside the SSA kernel; summed over devices for the
+ * multi-GPU combine (one ff_mapCUDA per GPU).  T = K+1 cuts, S species, B bins (all exact integers,
  * order-independent; a sum of buffers = the buffer of the union of instance ranges):
  *   [0, T)                       n[k]            instances present at cut k
  *   [T, T+TS)                    sum[k][s]       sum of x
  *   [T+TS, T+2TS)                sqlo[k][s]      sum of (x^2 mod 2^32)
  *   [T+2TS, T+3TS)               sqhi[k][s]      sum of (x^2 >> 32)       sum x^2 = sqhi*2^32 + sqlo
  *   [T+3TS, T+3TS+TS(B+2))       hist[k][s][b]   b=0 underflow, 1..B bins, B+1 overflow
- *   then 8 counters:             reactions, absorbed, overflowed, finished instances, 0...
+ *   then 8 counters:             reactions, absorbed, overflowed, finished instances, pool_full, 0...
+ *                                (pool_full: the overflowed instances frozen because a compartment pool
+ *                                was full, reading R20 — their later cuts are missing; a run with
+ *                                pool_full > 0 under-represents compartment-rich trajectories, so the
+ *                                Python API re-runs it with doubled capacities, see cwc_stats_t)
  */
 #define CWC_CTR_REACTIONS 0
 #define CWC_CTR_ABSORBED 1
 #define CWC_CTR_OVERFLOWED 2
 #define CWC_CTR_FINISHED 3
+#define CWC_CTR_POOL_FULL 4
 #define CWC_N_CTR 8
 /* With period analysis on ("period_species" >= 0), CWC_N_PERIOD arrays of T int64 follow the
  * counters: events, completed periods n / sum / sq_lo / sq_hi, local period n / sum / sq_lo /
@@ -245,7 +260,8 @@ cwc_status cwc_simulate_range(cwc_model_t m, int64_t n_total, int64_t first, int
 cwc_status cwc_stats_device(cwc_model_t m, int64_t** dptr, size_t* n_int64);
 
 /* Synchronise, copy the packed stats to the host and derive mean, variance (n-1; int128
- * numerator; NaN if n < 2) and inverted-CDF quantiles (R10, R11).  If host_stats is non-NULL
+ * numerator; NaN if n < 2) and inverted-CDF quantiles (R10, R11) — the "mean, variance" engines
+ * of the analysis stage.  If host_stats is non-NULL
  * the packed buffer is taken from it instead (e.g. after an NCCL all-reduce done by the
  * caller into host memory); it must hold stats_len int64 for the last simulated geometry. */
 cwc_status cwc_stats_finalize(cwc_model_t m, const int64_t* host_stats);
@@ -297,6 +313,8 @@ cwc_status cwc_stats_host(cwc_model_t m, const int64_t** host_stats, size_t* n_i
  * CWC_E_INVALID for a null buffer or cuts_final outside [0, T]. */
 cwc_status cwc_stats_load(cwc_model_t m, const int64_t* host_stats, int64_t cuts_final);
 
+/* The finalised statistics of every cut ("an array of results is produced and streamed
+ * to the analysis pipeline"; estimators P:L407; readings R10, R11, R14). */
 typedef struct {
     int32_t T, S, B, n_q;
     const double* times;      /* [T] t_k = fl(k*dt) */
@@ -316,6 +334,8 @@ typedef struct {
     double kernel_ms;         /* device time of the last simulate kernel (CUDA events) */
     int64_t cuts_final;       /* cuts [0, cuts_final) are final (T after finalize; see snapshot) */
     const char* const* species_names;
+    int64_t pool_full;        /* overflowed instances frozen by a full compartment pool (R20); 0 means
+                                 no trajectory was limited by a pool capacity */
 } cwc_stats_t;
 /* Borrowed views into the handle, valid until the next simulate / finalize / free. */
 cwc_status cwc_stats(cwc_model_t m, cwc_stats_t* out);
@@ -346,10 +366,14 @@ typedef struct {
 cwc_status cwc_period_stats(cwc_model_t m, cwc_period_stats_t* out);
 
 /* Raw samples of local instances [first, first+count) of the last simulated range, copied to
- * host out[T][S][count] (-1 = missing after an overflow).  CWC_E_STATE if raw_samples = 0. */
+ * host out[T][S][count] (-1 = missing after an overflow): the trajectory cuts themselves, "an
+ * array containing the results of all simulations at a given simulation time", per
+ * trajectory "the state of the system at each time step" sampled on the grid (R7).
+ * CWC_E_STATE if raw_samples = 0. */
 cwc_status cwc_samples(cwc_model_t m, int64_t first, int64_t count, int32_t* out);
 
-/* Per-instance records of the last simulated range (host outputs, any may be NULL):
+/* Per-instance records of the last simulated range (the simulation tasks' final state, P:L238-243;
+ * host outputs, any may be NULL):
  * flags (CWC_FLAG_*), reactions applied, final simulation time of the last applied reaction. */
 cwc_status cwc_instance_records(cwc_model_t m, int64_t first, int64_t count, uint8_t* flags,
                                 int64_t* reactions, double* t_last);

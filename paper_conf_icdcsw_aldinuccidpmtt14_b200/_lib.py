@@ -51,7 +51,8 @@ class Stats(ctypes.Structure):
                 ("sqlo", P(c_i64)), ("sqhi", P(c_i64)), ("mean", P(c_dbl)), ("var", P(c_dbl)),
                 ("hist", P(c_i64)), ("hist_lo", P(c_i64)), ("hist_width", P(c_i64)), ("q", P(c_dbl)),
                 ("quantile", P(c_dbl)), ("reactions", c_i64), ("absorbed", c_i64), ("overflowed", c_i64),
-                ("finished", c_i64), ("kernel_ms", c_dbl), ("cuts_final", c_i64), ("species_names", P(c_cp))]
+                ("finished", c_i64), ("kernel_ms", c_dbl), ("cuts_final", c_i64), ("species_names", P(c_cp)),
+                ("pool_full", c_i64)]
 
 
 class PeriodStats(ctypes.Structure):

@@ -61,6 +61,12 @@ class EnsembleResult:
     kernel_ms: float
     species: List[str]
     cuts_final: int = -1    # cuts [0, cuts_final) are final (T after finalize; a snapshot may be less)
+    pool_full: int = 0      # overflowed instances frozen by a full compartment pool (R20)
+
+    @property
+    def frozen_fraction(self) -> float:
+        """Fraction of the finished instances frozen before t_end (X_cap overflow or a full pool)."""
+        return self.overflowed / self.finished if self.finished else 0.0
 
     def sumsq_exact(self) -> np.ndarray:
         out = np.empty(self.sqlo.shape, dtype=object)
@@ -77,7 +83,8 @@ class Model:
                  quantiles: Optional[Sequence[float]] = None, raw_samples: bool = True,
                  quantum_samples: int = 0, block_threads: Optional[int] = None, refill: bool = True,
                  blocks_per_sm: int = 0, device: Optional[int] = None, period_species=None,
-                 period_lo: int = 0, period_hi: int = 1, period_window: int = 1, capacity=None, **options):
+                 period_lo: int = 0, period_hi: int = 1, period_window: int = 1, capacity=None,
+                 pool_auto: bool = True, **options):
         sp = (ctypes.c_char_p * len(species))(*[s.encode() for s in species])
         rl = (ctypes.c_char_p * max(len(rules), 1))(*[r.encode() for r in rules])
         rt = (ctypes.c_double * max(len(rates), 1))(*[float(k) for k in rates])
@@ -86,8 +93,22 @@ class Model:
         self._h = h
         self._info_cache = None
         self._bound_buffers = None   # DeviceBuffers bound to the handle (kept alive while bound)
-        for label, c in dict(capacity or {}).items():   # re-flattens: before species options (R20)
+        self._capacity = {k: int(v) for k, v in dict(capacity or {}).items()}
+        # reading R20': a simulation in which some instance found a compartment pool full is repeated
+        # with every pool capacity doubled (simulate / dist.simulate_sharded), until none is full
+        self.pool_auto = bool(pool_auto)
+        self._opts = dict(x_cap=x_cap, hist_bins=hist_bins, hist_width=hist_width, hist_lo=hist_lo,
+                          quantiles=quantiles, raw_samples=raw_samples, quantum_samples=quantum_samples,
+                          block_threads=block_threads, refill=refill, blocks_per_sm=blocks_per_sm, device=device,
+                          period_species=period_species, period_lo=period_lo, period_hi=period_hi,
+                          period_window=period_window, options=options)
+        for label, c in self._capacity.items():   # re-flattens: before species options (R20)
             self.set_option(f"capacity.{label}", int(c))
+        self._apply_options(**self._opts)
+
+    def _apply_options(self, *, x_cap, hist_bins, hist_width, hist_lo, quantiles, raw_samples, quantum_samples,
+                       block_threads, refill, blocks_per_sm, device, period_species, period_lo, period_hi,
+                       period_window, options):
         if x_cap is not None:
             self.set_option("x_cap", int(x_cap))
         if hist_bins is not None:
@@ -120,6 +141,26 @@ class Model:
             self.set_option("period_window", int(period_window))
         if device is not None:
             self.set_option("device", int(device))
+
+    # ------------------------------------------------------------ compartment pools (R20, R20')
+    def pool_capacities(self) -> dict:
+        """Slots per pool of every dynamic compartment label ({} for static models)."""
+        labels = sorted({n.split(":", 1)[1].split("@", 1)[0] for n in self.info()["names"] if n.startswith("#free:")})
+        return {lab: self._capacity.get(lab, 8) for lab in labels}
+
+    def grow_pools(self) -> bool:
+        """Double every pool capacity (max 4096), re-flatten and re-apply this model's options.
+        Returns False when no pool can grow (static model, or every pool at 4096 slots)."""
+        caps = self.pool_capacities()
+        grown = {lab: min(4096, 2 * c) for lab, c in caps.items()}
+        if not caps or grown == caps:
+            return False
+        for lab, c in grown.items():
+            self._capacity[lab] = c
+            self.set_option(f"capacity.{lab}", c)
+        self._info_cache = None
+        self._apply_options(**self._opts)
+        return True
 
     @classmethod
     def from_def(cls, mdef, **kw) -> "Model":
@@ -214,9 +255,14 @@ class Model:
 
     # ---------------------------------------------------------------- simulation
     def simulate(self, n_instances: int, t_end: float, sample_dt: float, seed: int) -> EnsembleResult:
-        """The public end-to-end call: simulate n instances, return host statistics."""
-        check(lib.cwc_simulate(self._h, int(n_instances), float(t_end), float(sample_dt), int(seed)))
-        return self.stats()
+        """The public end-to-end call: simulate n instances, return host statistics.  With
+        ``pool_auto`` (default) a run in which a compartment pool was full is repeated with doubled
+        pool capacities (reading R20'), so the result has pool_full == 0 unless a pool reached 4096."""
+        while True:
+            check(lib.cwc_simulate(self._h, int(n_instances), float(t_end), float(sample_dt), int(seed)))
+            res = self.stats()
+            if res.pool_full == 0 or not self.pool_auto or not self.grow_pools():
+                return res
 
     def simulate_range(self, n_total: int, first: int, count: int, t_end: float, sample_dt: float, seed: int,
                        stream=None) -> None:
@@ -253,7 +299,7 @@ class Model:
             quantile=arr(st.quantile, T * S * Q, np.float64, (T, S, Q)) if Q else np.zeros((T, S, 0)),
             reactions=st.reactions, absorbed=st.absorbed, overflowed=st.overflowed, finished=st.finished,
             kernel_ms=st.kernel_ms, species=[st.species_names[s].decode() for s in range(S)],
-            cuts_final=st.cuts_final,
+            cuts_final=st.cuts_final, pool_full=st.pool_full,
         )
 
     def snapshot(self):

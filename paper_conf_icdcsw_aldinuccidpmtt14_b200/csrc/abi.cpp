@@ -457,6 +457,7 @@ cwc_status cwc_stats(cwc_model_t m, cwc_stats_t* out) {
         out->absorbed = ctr[CWC_CTR_ABSORBED];
         out->overflowed = ctr[CWC_CTR_OVERFLOWED];
         out->finished = ctr[CWC_CTR_FINISHED];
+        out->pool_full = ctr[CWC_CTR_POOL_FULL];
         out->kernel_ms = m->kernel_ms;
         out->cuts_final = m->cuts_final;
         out->species_names = m->name_ptrs.data();

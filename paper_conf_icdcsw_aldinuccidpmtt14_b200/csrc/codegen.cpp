@@ -30,7 +30,8 @@ std::string generate_model_section(const FlatModel& fm, const KernelConfig& cfg)
       << "\n#define CWC_BLOCK " << cfg.block_threads << "\n#define CWC_MINB " << cfg.min_blocks << "\n#define CWC_ILP " << cfg.ilp << "\n";
     o << "#define CWC_PERIOD_S " << cfg.period_species << "\n#define CWC_PERIOD_LO " << cfg.period_lo
       << "LL\n#define CWC_PERIOD_HI " << cfg.period_hi << "LL\n";
-    o << "#define CWC_X_CAP " << cfg.x_cap << "\n#define CWC_FAST_CUT " << (cfg.fast_cut ? 1 : 0) << "\n\n";
+    o << "#define CWC_X_CAP " << cfg.x_cap << "\n#define CWC_FAST_CUT " << (cfg.fast_cut ? 1 : 0) << "\n";
+    o << "#define CWC_SENTINEL " << fm.sentinel << "  // species \"#full\" of the compartment pools (R20), -1 none\n\n";
     if (cfg.seed_keys) {
         const uint32_t k0 = (uint32_t)cfg.seed, k1 = (uint32_t)(cfg.seed >> 32);
         o << "#define CWC_STATIC_KEYS 1\nstatic constexpr cwc_round_keys cwc_rk_static = {{";

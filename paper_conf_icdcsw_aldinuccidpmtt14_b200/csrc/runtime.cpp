@@ -147,12 +147,24 @@ static std::string strip_pragma_once(const char* s) {
     return out;
 }
 
+// Development knob (same-box A/B of kernel revisions): CWC_DEVICE_SRC=<dir> compiles the device
+// sources cwc_params.h / cwc_rng.cuh / cwc_ssa.cuh found in <dir> instead of the embedded ones.
+static std::string device_source(const char* embedded, const char* file) {
+    const char* dir = std::getenv("CWC_DEVICE_SRC");
+    if (dir && *dir) {
+        std::ifstream f(std::string(dir) + "/" + file);
+        if (!f) fail(CWC_E_INVALID, std::string("CWC_DEVICE_SRC: cannot read ") + file);
+        return strip_pragma_once(std::string(std::istreambuf_iterator<char>(f), std::istreambuf_iterator<char>()).c_str());
+    }
+    return strip_pragma_once(embedded);
+}
+
 std::string generate_kernel_source(const FlatModel& fm, const KernelConfig& cfg) {
     std::string src = "// CWC ensemble SSA kernel, generated for one model (NVRTC, sm_100a)\n";
-    src += strip_pragma_once(cwc_embedded_params_h);
-    src += strip_pragma_once(cwc_embedded_rng_cuh);
+    src += device_source(cwc_embedded_params_h, "cwc_params.h");
+    src += device_source(cwc_embedded_rng_cuh, "cwc_rng.cuh");
     src += generate_model_section(fm, cfg);
-    src += strip_pragma_once(cwc_embedded_ssa_cuh);
+    src += device_source(cwc_embedded_ssa_cuh, "cwc_ssa.cuh");
     return src;
 }
 
@@ -219,15 +231,21 @@ static Nvrtc& nvrtc() {
 static const char* kNvrtcOpts[] = {"--gpu-architecture=sm_100a", "-fmad=false", "-lineinfo", "-std=c++17",
                                    "--ptxas-options=-v", "-DCWC_NVRTC=1"};
 
+// registers / spill stores of the SSA kernel itself (the module also holds the self-test kernel)
 static void parse_ptxas(cwc_model* m) {
     m->regs = -1;
     m->local_bytes = 0;
-    size_t p = m->nvrtc_log.find("Used ");
-    if (p != std::string::npos) m->regs = std::atoi(m->nvrtc_log.c_str() + p + 5);
-    size_t q = m->nvrtc_log.find("bytes spill stores");
-    if (q != std::string::npos) {
-        size_t b = m->nvrtc_log.rfind(',', q);
-        if (b != std::string::npos) m->local_bytes = std::atoi(m->nvrtc_log.c_str() + b + 1);
+    const std::string& log = m->nvrtc_log;
+    size_t start = log.find("entry function 'cwc_ssa_kernel'");
+    if (start == std::string::npos) start = 0;
+    size_t end = log.find("entry function", start + 1);
+    if (end == std::string::npos) end = log.size();
+    size_t p = log.find("Used ", start);
+    if (p != std::string::npos && p < end) m->regs = std::atoi(log.c_str() + p + 5);
+    size_t q = log.find("bytes spill stores", start);
+    if (q != std::string::npos && q < end) {
+        size_t b = log.rfind(',', q);
+        if (b != std::string::npos) m->local_bytes = std::atoi(log.c_str() + b + 1);
     }
 }
 

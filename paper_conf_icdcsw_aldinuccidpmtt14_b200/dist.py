@@ -61,10 +61,15 @@ class ShardedRun:
 
 
 def simulate_sharded(model, n_total: int, t_end: float, sample_dt: float, seed: int, group=None):
-    """Public multi-GPU call: every rank returns the statistics of the whole ensemble."""
-    run = ShardedRun(model, n_total, t_end, sample_dt, group)
-    run.launch(seed)
-    return run.result()
+    """Public multi-GPU call: every rank returns the statistics of the whole ensemble.  A run in
+    which some rank found a compartment pool full (pool_full counter of the all-reduced statistics:
+    the same on every rank) is repeated on every rank with doubled pool capacities (R20')."""
+    while True:
+        run = ShardedRun(model, n_total, t_end, sample_dt, group)
+        run.launch(seed)
+        res = run.result()
+        if res.pool_full == 0 or not getattr(model, "pool_auto", False) or not model.grow_pools():
+            return res
 
 
 _HOST_GROUPS = {}

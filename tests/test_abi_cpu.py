@@ -207,3 +207,25 @@ def test_steering_and_checkpoint_calls_out_of_order():
     with pytest.raises(cwc.CWCError) as e:
         m.restore(np.zeros(64, dtype=np.uint8))
     assert e.value.status == 1
+
+
+def test_pool_growth_reflattens_and_keeps_options():
+    """Reading R20': Model.grow_pools doubles every compartment-pool capacity, re-flattens the model
+    and re-applies the model's options (host only: flattening needs no GPU)."""
+    import dataclasses
+    import paper_conf_icdcsw_aldinuccidpmtt14_b200 as cwc
+    md = dataclasses.replace(W.VESICLES, capacity=(("ves", 3),))
+    m = cwc.Model.from_def(md, hist_bins=77, hist_width={"A": 2}, x_cap=5000)
+    assert m.pool_capacities() == {"ves": 3}
+    s3 = m.n_species
+    assert m.grow_pools() and m.pool_capacities() == {"ves": 6}
+    info = m.info()
+    assert m.n_species > s3 and sum(n.startswith("#alive") for n in info["names"]) == 6
+    assert info["hist_bins"] == 77 and info["x_cap"] == 5000
+    assert info["hist_width"][info["names"].index("A")] == 2
+    # the flat network at the grown capacity is the oracle's flattening at that capacity
+    from oracle.cwc_terms import flatten_def
+    fm = flatten_def(dataclasses.replace(md, capacity=(("ves", 6),)))
+    assert info["names"] == fm.names
+    static = cwc.Model.from_def(W.LOTKA_VOLTERRA)
+    assert static.pool_capacities() == {} and not static.grow_pools()

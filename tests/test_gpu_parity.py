@@ -469,3 +469,27 @@ def test_checkpoint_resume_with_period_analysis():
     for name in ("events", "pc_n", "pc_sum", "pc_sqlo", "pc_sqhi", "lp_n", "lp_sum", "lp_sqlo", "lp_sqhi"):
         assert np.array_equal(got[name], ref_p[name]), name
     assert np.array_equal(got["moving_avg"], ref_p["moving_avg"], equal_nan=True)
+
+
+def test_pool_auto_growth_removes_pool_frozen_instances():
+    """Reading R20': a run in which a compartment pool was full is repeated with doubled
+    capacities; the final result has no pool-frozen instance, and the species outside the pools
+    follow exactly the trajectories of an ample pool (the dynamics of a trajectory that never finds
+    its pool full do not depend on the capacity)."""
+    import dataclasses
+    import paper_conf_icdcsw_aldinuccidpmtt14_b200 as cwc
+    md = dataclasses.replace(W.VESICLES, capacity=(("ves", 3),))
+    n, t_end, dt, seed = 20_000, 60.0, 0.5, 11
+    m = cwc.Model.from_def(md, hist_bins=256)
+    m.pool_auto = False
+    first = m.simulate(n, t_end, dt, seed)
+    assert first.pool_full > 50 and first.pool_full <= first.overflowed     # capacity 3 fills often
+    m.pool_auto = True
+    res = m.simulate(n, t_end, dt, seed)
+    assert res.pool_full == 0 and m.pool_capacities()["ves"] >= 6
+    big = cwc.Model.from_def(dataclasses.replace(md, capacity=(("ves", 64),)), hist_bins=256).simulate(n, t_end, dt, seed)
+    assert big.pool_full == 0
+    for sp in ("A", "B", "C"):
+        i, j = res.species.index(sp), big.species.index(sp)
+        assert np.array_equal(res.sum[:, i], big.sum[:, j]) and np.array_equal(res.hist[:, i], big.hist[:, j]), sp
+    assert res.reactions == big.reactions and np.array_equal(res.n, big.n)
