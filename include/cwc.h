@@ -150,7 +150,9 @@ cwc_status cwc_model_info(cwc_model_t m, cwc_model_info_t* out);
  *   "hist_bins"          B >= 1 in-range bins per (time, species).               default 256
  *   "hist_width"         bin width >= 1 for every species;  "hist_width.<species name>" for one.
  *   "hist_lo"            left edge of bin 1 for every species; "hist_lo.<species name>" for one.
- *   "quantum_samples"    sample points per simulation quantum (Q/tau); 0 = auto.
+ *   "quantum_samples"    sample points per simulation quantum (Q/tau); 0 = auto:
+ *                        whole trajectories up to one instance per resident lane, else 32
+ *                        (up to 4 per lane) or 8 quanta, rounded up to a multiple of 8 cuts.
  *                        Scheduling only: results are bit-identical for every value (R12).
  *   "block_threads"      CUDA block size (multiple of 32, <= 1024).              default 768
  *   "blocks_per_sm"      persistent CTAs per SM; 0 = occupancy maximum.          default 0
@@ -167,6 +169,9 @@ cwc_status cwc_model_info(cwc_model_t m, cwc_model_info_t* out);
  *   "seed_jit"           0/1: specialise the kernel on the seed (Philox round keys become
  *                        instruction immediates; one NVRTC compile per new seed, cached).
  *   "refill"             0/1: warp-level refill from the global work queue.      default 1
+ *                        0 = static assignment: whole trajectories, or with quantum_samples > 0
+ *                        the paper's GPU scheme: one launch per simulation quantum,
+ *                        every lane running quantum q of its instance, launches as barriers.
  *   "device"             CUDA device ordinal.                                    default current
  * cwc_set_quantiles(m, n, q): quantile levels in [0,1] (R11), default {.05,.25,.5,.75,.95}.
  * Errors: CWC_E_INVALID (unknown key / bad value).

@@ -37,6 +37,7 @@ struct cwc_params {
     const cwc_logtab_entry* logtab;  // [128]
     long long smem_stats;       // 1: n/sum/sumsq accumulate per CTA in dynamic shared memory
                                 //    (T*(1+3S) u64) and are flushed once at the end
+    long long q0;               // quantum of work item 0 (per-quantum lockstep launches; else 0)
 };
 
 #define CWC_TERMINAL 0x80000000u

@@ -19,7 +19,7 @@
 #include <nvtx3/nvToolsExt.h>  // header-only NVTX v3: ranges are free unless a profiler injects
 
 // bench.py counts the launch parameter block in its end-to-end H2D bytes (PARAM_BYTES)
-static_assert(sizeof(cwc_params) == 248, "cwc_params layout changed: update bench.py PARAM_BYTES");
+static_assert(sizeof(cwc_params) == 256, "cwc_params layout changed: update bench.py PARAM_BYTES");
 static_assert(sizeof(cwc_logtab_entry) * 128 == 3072, "log table size");
 
 namespace {
@@ -503,6 +503,8 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     if (occ < 1) fail(CWC_E_CUDA, "kernel cannot be resident with block_threads = " + std::to_string(m->block_threads));
     size_t dyn_smem = 0;
     // streaming publishes partial statistics while the kernel runs: moments must go to global memory
+    // (a per-CTA shared-memory copy of the hottest histogram bin was measured slower: same-address
+    // shared atomics serialise too — vesicles 256 -> 273 ms, compartments 689 -> 728 ms)
     if (m->smem_stats && !m->stream && mom_bytes <= (size_t)200 * 1024) {
         ckd(d.FuncSetAttribute(m->function, CU_FUNC_ATTRIBUTE_MAX_DYNAMIC_SHARED_SIZE_BYTES, (int)mom_bytes),
             "dynamic smem");
@@ -519,10 +521,28 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     grid = std::min<int64_t>(grid, std::max<int64_t>(sms, (count + 32 * m->ilp - 1) / (32 * m->ilp)));
     const int64_t lanes = grid * m->block_threads * m->ilp;
     int64_t qs;
-    if (!m->refill) qs = T;  // static assignment: whole trajectories (no cross-lane dependencies)
+    // refill off: static assignment of whole trajectories, or — with quantum_samples set — the
+    // paper's GPU scheme: one launch per simulation quantum, every lane running its
+    // instance's quantum q, the kernel boundary as the barrier between quanta (the T3 ablation)
+    if (!m->refill) qs = m->quantum_samples > 0 ? std::min<int64_t>(m->quantum_samples, T) : T;
     else if (m->quantum_samples > 0) qs = std::min<int64_t>(m->quantum_samples, T);
     else if (m->stream) qs = std::max<int64_t>(1, (T + 15) / 16);  // streaming: progress in ~16 chunks
-    else qs = (count >= 4 * lanes) ? (T + 7) / 8 : T;
+    // auto (same-box sweeps, profiles/r2_ab_quanta_launch.log): up to one instance per resident lane, whole
+    // trajectories (a later quantum could only wait for its predecessor on another lane: LV 100k
+    // 1.37e11 whole vs 1.02e11 at 8 quanta); above, quanta let the surplus instances interleave with
+    // the first wave instead of forming a second one (LV 125k: 1.05e11 whole, 1.47e11 at 16 quanta,
+    // 1.57e11 at 32; LV 250k: 1.32e11 whole, 1.69e11 at 16-32); from 4 per lane the quantum count
+    // hardly matters (LV 1M: 1.701 / 1.711 / 1.706e11 at 32 / 16 / 8 quanta) and fewer quanta save
+    // state traffic (a save + restore per instance per quantum)
+    else if (count <= lanes) qs = T;
+    else {
+        // 32 quanta up to 4 instances per lane, 8 above; a quantum holds whole 8-cut blocks of the
+        // time-blocked raw layout, so each 32-byte sector is written by one lane in one quantum
+        // (no partially written sector left in L2 between quanta)
+        const int64_t nq_target = count <= 4 * lanes ? 32 : 8;
+        qs = (T + nq_target - 1) / nq_target;
+        qs = std::min<int64_t>(T, (qs + CWC_RAW_BLOCK - 1) / CWC_RAW_BLOCK * CWC_RAW_BLOCK);
+    }
     if (resume) qs = m->qs;  // the work items (quantum, instance) of the run being continued
     const int64_t nq = (T + qs - 1) / qs;
 
@@ -567,7 +587,12 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     }
     m->resumable = false;
     ck(cudaEventRecord(m->ev0, stream), "cudaEventRecord");
-    if (count > 0) {
+    const bool lockstep = !m->refill && qs < T;
+    for (int64_t q = 0; count > 0 && q < (lockstep ? nq : 1); ++q) {
+        if (lockstep) {  // quantum q only; the previous launch completed every quantum q-1 item
+            P.q0 = q;
+            P.n_items = count;
+        }
         void* args[] = {&P};
         ckd(d.LaunchKernel(m->function, (unsigned)grid, 1, 1, (unsigned)m->block_threads, 1, 1, (unsigned)dyn_smem,
                            (CUstream)stream,

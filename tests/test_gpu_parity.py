@@ -196,7 +196,8 @@ def test_schedule_invariance():
     base = None
     for opts in ({}, {"quantum_samples": 1}, {"quantum_samples": 7}, {"block_threads": 128},
                  {"fast_cut": 0}, {"fast_cut": 1, "quantum_samples": 3},
-                 {"block_threads": 512, "quantum_samples": 2}, {"refill": False}, {"blocks_per_sm": 1}):
+                 {"block_threads": 512, "quantum_samples": 2}, {"refill": False}, {"blocks_per_sm": 1},
+                 {"refill": False, "quantum_samples": 7}):   # per-quantum lockstep launches
         res, raw, flags, reactions, _ = gpu_run(md, 5000, 0, 5000, 4.0, 0.1, 42, hist_bins=512, **opts)
         cur = (res.n, res.sum, res.sqlo, res.sqhi, res.hist, raw, reactions)
         if base is None:

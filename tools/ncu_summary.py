@@ -12,7 +12,8 @@ KEYS = ["gpu__time_duration.sum", "sm__throughput.avg.pct_of_peak_sustained_elap
         "sm__inst_executed_pipe_lsu.avg.pct_of_peak_sustained_active",
         "sm__inst_executed_pipe_uniform.avg.pct_of_peak_sustained_active",
         "dram__bytes_read.sum", "dram__bytes_write.sum", "launch__registers_per_thread",
-        "launch__grid_size", "launch__occupancy_limit_registers", "sm__warps_active.avg.pct_of_peak_sustained_active"]
+        "launch__grid_size", "launch__occupancy_limit_registers", "sm__warps_active.avg.pct_of_peak_sustained_active",
+        "sm__pipe_fmaheavy_cycles_active.avg.pct_of_peak_sustained_active"]
 
 
 def main(path):
@@ -25,6 +26,10 @@ def main(path):
             print(f"{k:70s} {d[k][1]:>22s} {d[k][0]}")
     st = [(float(c.replace(',', '')), a) for a, b, c in zip(h, u, v)
           if a.startswith("smsp__average_warps_issue_stalled") and a.endswith("per_issue_active.ratio")]
+    if "smsp__inst_executed.sum" in d and "smsp__thread_inst_executed.sum" in d:
+        inst = float(d["smsp__inst_executed.sum"][1].replace(",", ""))
+        tinst = float(d["smsp__thread_inst_executed.sum"][1].replace(",", ""))
+        print(f"{'warp execution efficiency (thread_inst / (32 inst))':70s} {tinst / (32 * inst):>22.4f}")
     for val, name in sorted(st, reverse=True)[:8]:
         print(f"  stall {name.replace('smsp__average_warps_issue_stalled_', '').replace('_per_issue_active.ratio', ''):28s} {val:.3f}")
 
