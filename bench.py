@@ -41,7 +41,7 @@ import workloads as W  # noqa: E402
 
 METRIC = "simulated reactions/sec (whole box)"
 UNIT = "reactions/s"
-PARAM_BYTES = 256   # sizeof(cwc_params): the __grid_constant__ launch parameter block (static_assert in runtime.cpp)
+PARAM_BYTES = 272   # sizeof(cwc_params): the __grid_constant__ launch parameter block (static_assert in runtime.cpp)
 LOGTAB_BYTES = 3072  # CWC-log table uploaded once per model load (128 x {invc, logc, logclo})
 
 
@@ -379,10 +379,11 @@ def run_b200(args):
             "trajectories_per_s": traj_s,
             "reactions_per_step": total_reactions,
             "kernel_ms": kern_ms_max,
-            "gpu_launches": args.steps,
+            "gpu_launches": args.steps * res.launches,   # SSA (+ compaction) kernels of each step
             "roofline": roof,
             "cpu_baseline": cpu,
-            "e2e": {"value": e2e_value, "unit": UNIT, "h2d_bytes_per_step": PARAM_BYTES + LOGTAB_BYTES + cubin_bytes,
+            "e2e": {"value": e2e_value, "unit": UNIT,
+                    "h2d_bytes_per_step": PARAM_BYTES * r2.launches + LOGTAB_BYTES + cubin_bytes,
                     "d2h_bytes_per_step": n_stats * 8, "ms_per_step": float(te[0]),
                     "path": "Model.from_def + dist.simulate_sharded (public API): model load (host strings -> "
                             "flat model -> cached cubin -> module upload), buffers, launch + all-reduce, "

@@ -168,6 +168,11 @@ cwc_status cwc_model_info(cwc_model_t m, cwc_model_info_t* out);
  *                        Performance only: results are bit-identical.             default -1
  *   "seed_jit"           0/1: specialise the kernel on the seed (Philox round keys become
  *                        instruction immediates; one NVRTC compile per new seed, cached).
+ *   "compact"            0/1: compacted per-quantum launches — one launch per simulation quantum
+ *                        over the instances still running (a compaction kernel between launches),
+ *                        refill inside each launch (ablation: measured slower than the single
+ *                        persistent launch).  Scheduling only: results are bit-identical (R12).
+ *                                                                                   default 0
  *   "refill"             0/1: warp-level refill from the global work queue.      default 1
  *                        0 = static assignment: whole trajectories, or with quantum_samples > 0
  *                        the paper's GPU scheme: one launch per simulation quantum,
@@ -341,6 +346,7 @@ typedef struct {
     const char* const* species_names;
     int64_t pool_full;        /* overflowed instances frozen by a full compartment pool (R20); 0 means
                                  no trajectory was limited by a pool capacity */
+    int64_t launches;         /* kernels the last simulate launched (SSA + compaction) */
 } cwc_stats_t;
 /* Borrowed views into the handle, valid until the next simulate / finalize / free. */
 cwc_status cwc_stats(cwc_model_t m, cwc_stats_t* out);

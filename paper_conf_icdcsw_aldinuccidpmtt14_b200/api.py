@@ -62,6 +62,7 @@ class EnsembleResult:
     species: List[str]
     cuts_final: int = -1    # cuts [0, cuts_final) are final (T after finalize; a snapshot may be less)
     pool_full: int = 0      # overflowed instances frozen by a full compartment pool (R20)
+    launches: int = 1       # kernels the simulation launched (SSA + compaction)
 
     @property
     def frozen_fraction(self) -> float:
@@ -299,7 +300,7 @@ class Model:
             quantile=arr(st.quantile, T * S * Q, np.float64, (T, S, Q)) if Q else np.zeros((T, S, 0)),
             reactions=st.reactions, absorbed=st.absorbed, overflowed=st.overflowed, finished=st.finished,
             kernel_ms=st.kernel_ms, species=[st.species_names[s].decode() for s in range(S)],
-            cuts_final=st.cuts_final, pool_full=st.pool_full,
+            cuts_final=st.cuts_final, pool_full=st.pool_full, launches=st.launches,
         )
 
     def snapshot(self):

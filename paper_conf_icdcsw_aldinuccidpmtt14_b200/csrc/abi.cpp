@@ -275,6 +275,9 @@ cwc_status cwc_set_option_i64(cwc_model_t m, const char* key, int64_t v) {
         } else if (k == "refill") {
             need(v == 0 || v == 1, "refill is 0 or 1");
             m->refill = (int)v;
+        } else if (k == "compact") {
+            need(v == 0 || v == 1, "compact is 0 or 1");
+            m->compact = (int)v;
         } else if (k == "device") {
             need(v >= -1 && v < 1024, "bad device ordinal");
             m->device = (int)v;
@@ -458,6 +461,7 @@ cwc_status cwc_stats(cwc_model_t m, cwc_stats_t* out) {
         out->overflowed = ctr[CWC_CTR_OVERFLOWED];
         out->finished = ctr[CWC_CTR_FINISHED];
         out->pool_full = ctr[CWC_CTR_POOL_FULL];
+        out->launches = m->launches;
         out->kernel_ms = m->kernel_ms;
         out->cuts_final = m->cuts_final;
         out->species_names = m->name_ptrs.data();

@@ -37,7 +37,11 @@ struct cwc_params {
     const cwc_logtab_entry* logtab;  // [128]
     long long smem_stats;       // 1: n/sum/sumsq accumulate per CTA in dynamic shared memory
                                 //    (T*(1+3S) u64) and are flushed once at the end
-    long long q0;               // quantum of work item 0 (per-quantum lockstep launches; else 0)
+    long long q0;               // quantum of work item 0 (per-quantum launches; else 0)
+    // compacted per-quantum launches: work item w is quantum q0 of local instance list[w]; the
+    // item count is *n_items_dev (written by the previous launch's compaction), else n_items
+    const unsigned int* list;
+    const unsigned long long* n_items_dev;
 };
 
 #define CWC_TERMINAL 0x80000000u

@@ -19,7 +19,7 @@
 #include <nvtx3/nvToolsExt.h>  // header-only NVTX v3: ranges are free unless a profiler injects
 
 // bench.py counts the launch parameter block in its end-to-end H2D bytes (PARAM_BYTES)
-static_assert(sizeof(cwc_params) == 256, "cwc_params layout changed: update bench.py PARAM_BYTES");
+static_assert(sizeof(cwc_params) == 272, "cwc_params layout changed: update bench.py PARAM_BYTES");
 static_assert(sizeof(cwc_logtab_entry) * 128 == 3072, "log table size");
 
 namespace {
@@ -111,7 +111,7 @@ size_t stats_len(int64_t T, int S, int B, bool period) {
 static size_t align256(size_t v) { return (v + 255) & ~(size_t)255; }
 
 struct ScratchLayout {
-    size_t x, t, step, k, flags, pd, qdone, work, cancel, qprog, total;
+    size_t x, t, step, k, flags, pd, qdone, work, cancel, qprog, list0, list1, nlive, total;
 };
 
 static ScratchLayout scratch_layout(int S, int64_t count, int64_t T) {
@@ -128,6 +128,9 @@ static ScratchLayout scratch_layout(int S, int64_t count, int64_t T) {
     L.work = off; off += 8;
     L.cancel = off; off += 8;                         // u32 terminate flag (streaming)
     L.qprog = off; off = align256(off + (size_t)T * 4);  // <= T quanta
+    L.list0 = off; off = align256(off + (size_t)count * 4);  // compacted launches: running instances
+    L.list1 = off; off = align256(off + (size_t)count * 4);
+    L.nlive = off; off = align256(off + 16);                 // their counts (two u64)
     L.total = off;
     return L;
 }
@@ -367,6 +370,7 @@ static void ensure_module(cwc_model* m, int dev) {
     m->module = nullptr;
     ckd(d.ModuleLoadData(&m->module, m->cubin.data()), "cuModuleLoadData");
     ckd(d.ModuleGetFunction(&m->function, m->module, "cwc_ssa_kernel"), "cuModuleGetFunction");
+    ckd(d.ModuleGetFunction(&m->compact_fn, m->module, "cwc_compact_kernel"), "cuModuleGetFunction(compact)");
     m->module_device = dev;
     int v = 0;
     if (d.FuncGetAttribute(&v, CU_FUNC_ATTRIBUTE_NUM_REGS, m->function) == CUDA_SUCCESS) m->regs = v;
@@ -524,8 +528,15 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     // refill off: static assignment of whole trajectories, or — with quantum_samples set — the
     // paper's GPU scheme: one launch per simulation quantum, every lane running its
     // instance's quantum q, the kernel boundary as the barrier between quanta (the T3 ablation)
+    // compacted launches (option; ablation of the under-filled regime): a quantum per launch over
+    // the instances still running, so the lanes of instances that ended are handed back at every
+    // launch instead of idling to the end — measured slower than one persistent launch
+    const bool compact = m->refill && !m->stream && !resume && count > 0 && m->compact == 1;
     if (!m->refill) qs = m->quantum_samples > 0 ? std::min<int64_t>(m->quantum_samples, T) : T;
-    else if (m->quantum_samples > 0) qs = std::min<int64_t>(m->quantum_samples, T);
+    else if (compact) {
+        qs = m->quantum_samples > 0 ? std::min<int64_t>(m->quantum_samples, T) : (T + 7) / 8;
+        qs = std::min<int64_t>(T, (qs + CWC_RAW_BLOCK - 1) / CWC_RAW_BLOCK * CWC_RAW_BLOCK);
+    } else if (m->quantum_samples > 0) qs = std::min<int64_t>(m->quantum_samples, T);
     else if (m->stream) qs = std::max<int64_t>(1, (T + 15) / 16);  // streaming: progress in ~16 chunks
     // auto (same-box sweeps, profiles/r2_ab_quanta_launch.log): up to one instance per resident lane, whole
     // trajectories (a later quantum could only wait for its predecessor on another lane: LV 100k
@@ -588,16 +599,40 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     m->resumable = false;
     ck(cudaEventRecord(m->ev0, stream), "cudaEventRecord");
     const bool lockstep = !m->refill && qs < T;
-    for (int64_t q = 0; count > 0 && q < (lockstep ? nq : 1); ++q) {
-        if (lockstep) {  // quantum q only; the previous launch completed every quantum q-1 item
+    const bool per_quantum = (lockstep || compact) && nq > 1;
+    unsigned int* lists[2] = {(unsigned int*)(sc + L.list0), (unsigned int*)(sc + L.list1)};
+    unsigned long long* nlive = (unsigned long long*)(sc + L.nlive);
+    m->launches = 0;
+    for (int64_t q = 0; count > 0 && q < (per_quantum ? nq : 1); ++q) {
+        if (per_quantum) {  // quantum q only; the previous launch completed every quantum q-1 item
             P.q0 = q;
             P.n_items = count;
+        }
+        if (compact && q > 0) {  // the instances still running after quantum q-1
+            P.list = lists[(q - 1) & 1];
+            P.n_items_dev = nlive + ((q - 1) & 1);
+            ck(cudaMemsetAsync(P.work, 0, 8, stream), "memset(work)");
         }
         void* args[] = {&P};
         ckd(d.LaunchKernel(m->function, (unsigned)grid, 1, 1, (unsigned)m->block_threads, 1, 1, (unsigned)dyn_smem,
                            (CUstream)stream,
                            args, nullptr),
             "cuLaunchKernel");
+        ++m->launches;
+        if (compact && q + 1 < nq) {
+            unsigned long long* n_out = nlive + (q & 1);
+            ck(cudaMemsetAsync(n_out, 0, 8, stream), "memset(nlive)");
+            const unsigned int* l_in = q > 0 ? lists[(q - 1) & 1] : nullptr;
+            const unsigned long long* n_in_dev = q > 0 ? nlive + ((q - 1) & 1) : nullptr;
+            unsigned long long n_in = (unsigned long long)count;
+            const unsigned int* flags = (const unsigned int*)P.st_flags;
+            unsigned int* l_out = lists[q & 1];
+            void* cargs[] = {(void*)&l_in, (void*)&n_in_dev, &n_in, (void*)&flags, &l_out, &n_out};
+            const unsigned cgrid = (unsigned)std::min<int64_t>((count + 255) / 256, (int64_t)sms * 8);
+            ckd(d.LaunchKernel(m->compact_fn, cgrid, 1, 1, 256, 1, 1, 0, (CUstream)stream, cargs, nullptr),
+                "cuLaunchKernel(compact)");
+            ++m->launches;
+        }
     }
     ck(cudaEventRecord(m->ev1, stream), "cudaEventRecord");
     ck(cudaGetLastError(), "launch");

@@ -49,6 +49,13 @@ struct cwc_model {
     int64_t cuts_final = 0;               // cuts final in the host views (T after finalize)
     int blocks_per_sm = 0;
     int refill = 1;
+    // compacted per-quantum launches (0 off, 1 on): one launch per quantum over the instances
+    // still running, refill inside the launch, a compaction kernel between launches.  Measured
+    // slower than the single persistent launch in the under-filled regime it targets (the launch
+    // boundaries cost more than the handed-back lanes gain: LV 100k 1.41e11 -> 1.21e11,
+    // profiles/r2_ab_quanta_launch.log), so an ablation mode only
+    int compact = 0;
+    int launches = 0;                     // SSA + compaction kernels of the last simulate
     int device = -1;
     std::vector<double> quantiles{0.05, 0.25, 0.5, 0.75, 0.95};
 
@@ -64,6 +71,7 @@ struct cwc_model {
     int regs = -1, local_bytes = -1, max_threads = -1;
     CUmodule module = nullptr;
     CUfunction function = nullptr;
+    CUfunction compact_fn = nullptr;
     int module_device = -1;
 
     // device buffers (owned or bound)

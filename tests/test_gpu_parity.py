@@ -104,6 +104,16 @@ def test_terminated_instances_under_quanta():
     assert res.overflowed > 0 and res.absorbed > 0
 
 
+@pytest.mark.parametrize("q", [0, 16])
+def test_compacted_launches_drop_finished_instances(q):
+    """Compacted per-quantum launches (option compact): instances that absorb or overflow leave
+    the launch lists; every instance's cuts, flags and reactions still equal the oracle's."""
+    cfg = W.CONFIGS["lv"]
+    res, raw, m = _parity(cfg.model, 700, 50.0, 0.5, cfg.seed + 7, hist_bins=cfg.hist_bins,
+                          hist_width=cfg.hist_width, compact=1, quantum_samples=q)
+    assert res.overflowed > 0 and res.absorbed > 0 and res.launches > 2
+
+
 def test_lv_long_horizon_absorb_and_overflow():
     # long horizon: predator extinction, prey runaway past X_cap (R9) and full extinction (R8)
     cfg = W.CONFIGS["lv"]
@@ -197,7 +207,8 @@ def test_schedule_invariance():
     for opts in ({}, {"quantum_samples": 1}, {"quantum_samples": 7}, {"block_threads": 128},
                  {"fast_cut": 0}, {"fast_cut": 1, "quantum_samples": 3},
                  {"block_threads": 512, "quantum_samples": 2}, {"refill": False}, {"blocks_per_sm": 1},
-                 {"refill": False, "quantum_samples": 7}):   # per-quantum lockstep launches
+                 {"refill": False, "quantum_samples": 7},    # per-quantum lockstep launches
+                 {"compact": 1}, {"compact": 1, "quantum_samples": 3}, {"compact": 0}):  # compacted launches
         res, raw, flags, reactions, _ = gpu_run(md, 5000, 0, 5000, 4.0, 0.1, 42, hist_bins=512, **opts)
         cur = (res.n, res.sum, res.sqlo, res.sqhi, res.hist, raw, reactions)
         if base is None:

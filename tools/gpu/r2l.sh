@@ -16,3 +16,6 @@ prof neurospora neurospora 1000000 raw=0
 prof vesicles vesicles 1000000 raw=0
 prof lv100k lv 100000
 prof lv125k lv 125000
+for c in lv schlogl circadian compartments neurospora vesicles; do timeout 300 python tools/imin.py $c > /dev/null 2>&1; done
+cp profiles/imin_*.json gpurun_out/
+cat profiles/imin_*.json
