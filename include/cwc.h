@@ -231,7 +231,7 @@ cwc_status cwc_bind_device_buffers(cwc_model_t m, int64_t* stats, size_t stats_l
  * (cwc_stats_finalize / cwc_samples / cwc_instance_records synchronise it).
  * cwc_simulate(m, n, t_end, dt, seed) == cwc_simulate_range(m, n, 0, n, ...) on the handle's
  * own stream followed by cwc_stats_finalize (synchronous).
- * Errors: CWC_E_INVALID (n_total <= 0, count < 0, first+count > n_total, t_end < 0,
+ * Errors: CWC_E_INVALID (n_total <= 0, count < 0, first+count > n_total, count >= 2^31, t_end < 0,
  *         sample_dt <= 0, |K*dt - t_end| > 1e-9*max(1,t_end), buffers too small);
  *         CWC_E_OOM; CWC_E_CUDA.
  * ---------------------------------------------------------------------------------------- */

@@ -68,9 +68,12 @@ std::string generate_model_section(const FlatModel& fm, const KernelConfig& cfg)
     }
     for (int s = 0; s < S; ++s) {
         if (need[s][1] || need[s][2]) o << "    const double f" << s << "_1 = (double)x[" << s << "];\n";
+        // C(x, 2) = x (x - 1) / 2: x - 1 as an exact DADD (no second conversion); x (x - 1) is an
+        // even integer < 2^54, exact in a double, and so is its half (x = 0 gives -0.0, which every
+        // use treats as 0: a_j = +-0, cum unchanged, never selected)
         if (need[s][2])
-            o << "    const double f" << s << "_2 = __dmul_rn(__dmul_rn(f" << s << "_1, (double)(x[" << s << "] > 0 ? x["
-              << s << "] - 1 : 0)), 0.5);\n";
+            o << "    const double f" << s << "_2 = __dmul_rn(__dmul_rn(f" << s << "_1, __dsub_rn(f" << s
+              << "_1, 1.0)), 0.5);\n";
         if (need[s][3])
             o << "    const double f" << s << "_3 = (double)(((long long)x[" << s << "] * (long long)(x[" << s
               << "] - 1) / 2) * (long long)(x[" << s << "] - 2) / 3);\n";

@@ -458,6 +458,7 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     NvtxRange nvtx_range("cwc_simulate_range");
     if (n_total <= 0) fail(CWC_E_INVALID, "n_total must be > 0");
     if (first < 0 || count < 0 || first + count > n_total) fail(CWC_E_INVALID, "instance range outside [0, n_total)");
+    if (count >= ((int64_t)1 << 31)) fail(CWC_E_INVALID, "at most 2^31 - 1 instances per range (shard larger ensembles)");
     const int64_t K = grid_K(t_end, dt);
     if (m->period_species >= 0 && !(m->period_lo < m->period_hi))
         fail(CWC_E_INVALID, "period analysis needs period_lo < period_hi");
@@ -1041,7 +1042,8 @@ struct SelftestIo {  // mirrors cwc_selftest_io (cwc_ssa.cuh)
 void selftest_step(cwc_model* m, int64_t n, int32_t n_draws, const int32_t* x, const double* t, const int64_t* k,
                    double t_end, double dt, const double* u_tau, const double* u_sel, int32_t mode, int32_t* x_out,
                    double* t_out, int64_t* k_out, int32_t* status, int32_t* n_done, int32_t* cuts) {
-    if (n < 0 || n_draws < 1 || (mode != 0 && mode != 1)) fail(CWC_E_INVALID, "bad self-test arguments");
+    if (n < 0 || n >= ((int64_t)1 << 31) || n_draws < 1 || (mode != 0 && mode != 1))
+        fail(CWC_E_INVALID, "bad self-test arguments");
     const int64_t K = grid_K(t_end, dt), T = K + 1;
     const int S = m->fm.S();
     for (int64_t i = 0; i < n; ++i)
