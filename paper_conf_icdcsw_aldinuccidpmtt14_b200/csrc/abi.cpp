@@ -255,7 +255,7 @@ cwc_status cwc_set_option_i64(cwc_model_t m, const char* key, int64_t v) {
             need(v == 0 || v == 1, "stream is 0 or 1");
             m->stream = (int)v;
         } else if (k == "smem_stats") {
-            need(v == 0 || v == 1, "smem_stats is 0 or 1");
+            need(v >= 0 && v <= 3, "smem_stats is 0 (global), 1 (auto), 2 (sparse) or 3 (dense)");
             m->smem_stats = (int)v;
         } else if (k == "ilp") {
             need(v == 1 || v == 2, "ilp is 1 or 2");

@@ -18,6 +18,14 @@
 #include <dlfcn.h>
 #include <nvtx3/nvToolsExt.h>  // header-only NVTX v3: ranges are free unless a profiler injects
 
+// models with at least this many species accumulate cut statistics in the sparse shared layout
+// (same-box A/B, profiles/r2_ab_kernel.log, sparse vs dense: vesicles 123 vs 228 ms, compartments
+// 625 vs 686, Neurospora 653 vs 684, circadian 1750 vs 1794, Schlogl 1916 vs 1953, LV 1M 1717 vs
+// 1725: every model)
+#ifndef CWC_SPARSE_MIN_S
+#define CWC_SPARSE_MIN_S 1
+#endif
+
 // bench.py counts the launch parameter block in its end-to-end H2D bytes (PARAM_BYTES)
 static_assert(sizeof(cwc_params) == 272, "cwc_params layout changed: update bench.py PARAM_BYTES");
 static_assert(sizeof(cwc_logtab_entry) * 128 == 3072, "log table size");
@@ -507,15 +515,29 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     ckd(d.Occupancy(&occ, m->function, m->block_threads, 0), "occupancy");
     if (occ < 1) fail(CWC_E_CUDA, "kernel cannot be resident with block_threads = " + std::to_string(m->block_threads));
     size_t dyn_smem = 0;
-    // streaming publishes partial statistics while the kernel runs: moments must go to global memory
-    // (a per-CTA shared-memory copy of the hottest histogram bin was measured slower: same-address
-    // shared atomics serialise too — vesicles 256 -> 273 ms, compartments 689 -> 728 ms)
-    if (m->smem_stats && !m->stream && mom_bytes <= (size_t)200 * 1024) {
-        ckd(d.FuncSetAttribute(m->function, CU_FUNC_ATTRIBUTE_MAX_DYNAMIC_SHARED_SIZE_BYTES, (int)mom_bytes),
+    int smem_mode = 0;
+    // Per-CTA shared-memory accumulators when they fit without lowering residency: sparse (u32
+    // counters and 16-bit limbs with native shared REDs, zero counts skipped and restored at the
+    // flush) or dense (u64 n / sum / sum-of-squares halves: 64-bit shared atomics are CAS loops).  Streaming publishes partial
+    // statistics while the kernel runs, so it keeps everything in global memory.  (A per-CTA copy
+    // of the hottest histogram bin alone was measured slower: vesicles 256 -> 273 ms.)
+    const size_t sparse_bytes = (size_t)T * (1 + 7 * (size_t)S) * 4;
+    auto fits = [&](size_t bytes) {
+        if (bytes > (size_t)200 * 1024) return false;
+        ckd(d.FuncSetAttribute(m->function, CU_FUNC_ATTRIBUTE_MAX_DYNAMIC_SHARED_SIZE_BYTES, (int)bytes),
             "dynamic smem");
         int occ2 = 0;
-        ckd(d.Occupancy(&occ2, m->function, m->block_threads, mom_bytes), "occupancy");
-        if (occ2 >= occ) dyn_smem = mom_bytes;
+        ckd(d.Occupancy(&occ2, m->function, m->block_threads, bytes), "occupancy");
+        return occ2 >= occ;
+    };
+    if (m->smem_stats && !m->stream) {
+        // sparse limbs need < 65537 cuts of one (cut, species) per CTA: at most 65536 instances per CTA
+        const bool sparse_ok = count <= (int64_t)65536 * sms;
+        const bool want_sparse = sparse_ok && (m->smem_stats == 2 || (m->smem_stats == 1 && S >= CWC_SPARSE_MIN_S));
+        if (want_sparse && fits(sparse_bytes)) smem_mode = 2, dyn_smem = sparse_bytes;
+        else if (m->smem_stats != 2 && fits(mom_bytes)) smem_mode = 1, dyn_smem = mom_bytes;
+        ckd(d.FuncSetAttribute(m->function, CU_FUNC_ATTRIBUTE_MAX_DYNAMIC_SHARED_SIZE_BYTES, (int)dyn_smem),
+            "dynamic smem");
     }
     int per_sm = m->blocks_per_sm > 0 ? std::min(m->blocks_per_sm, occ) : occ;
     int64_t grid = (int64_t)sms * per_sm;
@@ -589,7 +611,7 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     P.cancel = m->stream ? (const unsigned int*)(sc + L.cancel) : nullptr;
     m->cancel_requested = false;
     P.logtab = m->d_logtab;
-    P.smem_stats = dyn_smem ? 1 : 0;
+    P.smem_stats = smem_mode;
 
     if (!resume) {
         ck(cudaMemsetAsync(m->d_stats, 0, need_stats * 8, stream), "memset(stats)");

@@ -218,6 +218,28 @@ def test_schedule_invariance():
                 assert np.array_equal(a, b), opts
 
 
+@pytest.mark.parametrize("name,n", [("circadian", 3000), ("vesicles", 3000), ("lv", 2000), ("schlogl", 3000)])
+def test_statistics_staging_invariance(name, n):
+    """The three per-CTA staging layouts of the cut statistics (global only, sparse u32 limbs with
+    zero counts restored at the flush, dense u64) give bit-identical packed statistics, and the
+    default one equals the oracle's statistics of its own samples."""
+    cfg = W.CONFIGS[name]
+    t_end = min(cfg.t_end, 10.0)
+    base = None
+    for mode in (0, 1, 2, 3):
+        res, raw, *_ = gpu_run(cfg.model, n, 0, n, t_end, cfg.sample_dt, cfg.seed, hist_bins=cfg.hist_bins,
+                               hist_width=cfg.hist_width, smem_stats=mode)
+        cur = (res.n, res.sum, res.sqlo, res.sqhi, res.hist, res.reactions)
+        if base is None:
+            base = cur
+            orun = _oracle(cfg.model, 0, n, t_end, cfg.sample_dt, cfg.seed)
+            assert np.array_equal(raw, orun.raw)
+            assert_matches_oracle_stats(res, orun.raw, QS)
+        else:
+            for a, b in zip(base, cur):
+                assert np.array_equal(a, b), mode
+
+
 def test_sharding_invariance():
     """Disjoint ranges summed == one run (what the NCCL all-reduce relies on, §8(e))."""
     md, N, t_end, dt, seed = W.LOTKA_VOLTERRA, 4000, 3.0, 0.1, 7
