@@ -165,7 +165,7 @@ cwc_status cwc_model_info(cwc_model_t m, cwc_model_info_t* out);
  *                        16-bit limbs, zero counts restored at the flush; T*(1+7S)*4 bytes); 3
  *                        dense per-CTA shared moments (u64, T*(1+3S)*8 bytes); 1 auto = sparse,
  *                        else dense, else global — each only when it fits without lowering
- *                        residency (sparse: at most 65536 instances per SM).  Bit-identical.  default 1
+ *                        residency.  Results are bit-identical.                  default 1
  *   "fast_cut"           -1/0/1: where cuts are recorded — inside the fast step (1) or on the
  *                        full-step path (0); -1 = auto: 0 when the last simulation on this handle
  *                        (else a0(x0)*sample_dt) had >= 1000 reactions per recorded cut.

@@ -521,7 +521,7 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     // flush) or dense (u64 n / sum / sum-of-squares halves: 64-bit shared atomics are CAS loops).  Streaming publishes partial
     // statistics while the kernel runs, so it keeps everything in global memory.  (A per-CTA copy
     // of the hottest histogram bin alone was measured slower: vesicles 256 -> 273 ms.)
-    const size_t sparse_bytes = (size_t)T * (1 + 7 * (size_t)S) * 4;
+    const size_t sparse_bytes = (size_t)T * (2 + 7 * (size_t)S) * 4;  // counters + per-quantum admissions
     auto fits = [&](size_t bytes) {
         if (bytes > (size_t)200 * 1024) return false;
         ckd(d.FuncSetAttribute(m->function, CU_FUNC_ATTRIBUTE_MAX_DYNAMIC_SHARED_SIZE_BYTES, (int)bytes),
@@ -531,9 +531,9 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
         return occ2 >= occ;
     };
     if (m->smem_stats && !m->stream) {
-        // sparse limbs need < 65537 cuts of one (cut, species) per CTA: at most 65536 instances per CTA
-        const bool sparse_ok = count <= (int64_t)65536 * sms;
-        const bool want_sparse = sparse_ok && (m->smem_stats == 2 || (m->smem_stats == 1 && S >= CWC_SPARSE_MIN_S));
+        // (the sparse limbs are exact for any count: a CTA's records beyond 65536 per cut index go to
+        // global memory directly)
+        const bool want_sparse = m->smem_stats == 2 || (m->smem_stats == 1 && S >= CWC_SPARSE_MIN_S);
         if (want_sparse && fits(sparse_bytes)) smem_mode = 2, dyn_smem = sparse_bytes;
         else if (m->smem_stats != 2 && fits(mom_bytes)) smem_mode = 1, dyn_smem = mom_bytes;
         ckd(d.FuncSetAttribute(m->function, CU_FUNC_ATTRIBUTE_MAX_DYNAMIC_SHARED_SIZE_BYTES, (int)dyn_smem),

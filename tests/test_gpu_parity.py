@@ -240,6 +240,21 @@ def test_statistics_staging_invariance(name, n):
                 assert np.array_equal(a, b), mode
 
 
+def test_sparse_ticket_overflow_goes_global(monkeypatch):
+    """Sparse staging admits at most CWC_SPARSE_TICKETS work items of one quantum per CTA to its
+    16-bit limbs; later items record to global memory.  With the limit lowered to 64 most records
+    take that path, and the statistics still equal the oracle's (and the default kernel's)."""
+    cfg = W.CONFIGS["compartments"]
+    n, t_end = 20_000, 10.0
+    ref, *_ = gpu_run(cfg.model, n, 0, n, t_end, cfg.sample_dt, cfg.seed, hist_bins=cfg.hist_bins, raw=False)
+    monkeypatch.setenv("CWC_KERNEL_DEFINES", "CWC_SPARSE_TICKETS=64")
+    res, raw, *_ = gpu_run(cfg.model, n, 0, n, t_end, cfg.sample_dt, cfg.seed, hist_bins=cfg.hist_bins,
+                           smem_stats=2)
+    for name in ("n", "sum", "sqlo", "sqhi", "hist"):
+        assert np.array_equal(getattr(res, name), getattr(ref, name)), name
+    assert_matches_oracle_stats(res, _oracle(cfg.model, 0, n, t_end, cfg.sample_dt, cfg.seed).raw, QS)
+
+
 def test_sharding_invariance():
     """Disjoint ranges summed == one run (what the NCCL all-reduce relies on, §8(e))."""
     md, N, t_end, dt, seed = W.LOTKA_VOLTERRA, 4000, 3.0, 0.1, 7
