@@ -27,6 +27,10 @@ def main():
         (W.NEUROSPORA, 200, 6.0, 0.5, {"period_species": "M", "period_lo": 100, "period_hi": 350}),
         (W.RUNAWAY, 100, 10.0, 0.5, {}),
         (W.DEAD, 100, 3.0, 0.5, {}),
+        # round 2: dense staging, compacted per-quantum launches, the paper's lockstep launches
+        (W.COMPARTMENTS, 200, 2.0, 0.5, {"smem_stats": 3}),
+        (W.LOTKA_VOLTERRA, 300, 0.3, 0.05, {"compact": 1, "quantum_samples": 2}),
+        (W.SCHLOGL, 500, 0.5, 0.05, {"refill": False, "quantum_samples": 3}),
     ]
     for md, n, t_end, dt, opts in runs:
         m = cwc.Model.from_def(md, hist_bins=64, **opts)
@@ -59,6 +63,19 @@ def main():
     res = m2.finalize()
     assert res.finished == 4000
     print(f"checkpoint/resume ok (cuts final at stop {cf})", flush=True)
+    # sparse staging with most items over the admission limit (the global overflow path)
+    os.environ["CWC_KERNEL_DEFINES"] = "CWC_SPARSE_TICKETS=4"
+    m = cwc.Model.from_def(W.CIRCADIAN, hist_bins=64, smem_stats=2)
+    assert m.simulate(400, 4.0, 0.5, 13).finished == 400
+    del os.environ["CWC_KERNEL_DEFINES"]
+    print("sparse admission overflow ok", flush=True)
+    # the injected-draw self-test kernel (both modes)
+    m = cwc.Model.from_def(W.LOTKA_VOLTERRA, hist_bins=64)
+    for mode in (0, 1):
+        out = m.selftest_step([[1000, 1000]] * 64, [0.0] * 64, [1] * 64, 1.0, 0.1, [[0.5] * 8] * 64, [[0.3] * 8] * 64,
+                              mode=mode)
+        assert (out["n_done"] >= 1).all()
+    print("self-test step ok", flush=True)
 
 
 if __name__ == "__main__":
