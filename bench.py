@@ -41,7 +41,7 @@ import workloads as W  # noqa: E402
 
 METRIC = "simulated reactions/sec (whole box)"
 UNIT = "reactions/s"
-PARAM_BYTES = 272   # sizeof(cwc_params): the __grid_constant__ launch parameter block (static_assert in runtime.cpp)
+PARAM_BYTES = 280   # sizeof(cwc_params): the __grid_constant__ launch parameter block (static_assert in runtime.cpp)
 LOGTAB_BYTES = 3072  # CWC-log table uploaded once per model load (128 x {invc, logc, logclo})
 
 

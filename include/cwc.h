@@ -166,6 +166,10 @@ cwc_status cwc_model_info(cwc_model_t m, cwc_model_info_t* out);
  *                        dense per-CTA shared moments (u64, T*(1+3S)*8 bytes); 1 auto = sparse,
  *                        else dense, else global — each only when it fits without lowering
  *                        residency.  Results are bit-identical.                  default 1
+ *   "raw_stage"          0/1: a lane collects the 8 cuts of one 32-byte block of the raw layout in
+ *                        shared memory and writes the block as whole sectors (1: when it fits
+ *                        without lowering residency and ilp = 1).  Results are bit-identical.
+ *                                                                                   default 1
  *   "fast_cut"           -1/0/1: where cuts are recorded — inside the fast step (1) or on the
  *                        full-step path (0); -1 = auto: 0 when the last simulation on this handle
  *                        (else a0(x0)*sample_dt) had >= 1000 reactions per recorded cut.
@@ -351,6 +355,7 @@ typedef struct {
     int64_t pool_full;        /* overflowed instances frozen by a full compartment pool (R20); 0 means
                                  no trajectory was limited by a pool capacity */
     int64_t launches;         /* kernels the last simulate launched (SSA + compaction) */
+    int64_t raw_staged;       /* 1: the last simulate staged raw cuts in shared memory (raw_stage) */
 } cwc_stats_t;
 /* Borrowed views into the handle, valid until the next simulate / finalize / free. */
 cwc_status cwc_stats(cwc_model_t m, cwc_stats_t* out);

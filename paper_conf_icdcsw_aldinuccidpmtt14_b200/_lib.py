@@ -52,7 +52,7 @@ class Stats(ctypes.Structure):
                 ("hist", P(c_i64)), ("hist_lo", P(c_i64)), ("hist_width", P(c_i64)), ("q", P(c_dbl)),
                 ("quantile", P(c_dbl)), ("reactions", c_i64), ("absorbed", c_i64), ("overflowed", c_i64),
                 ("finished", c_i64), ("kernel_ms", c_dbl), ("cuts_final", c_i64), ("species_names", P(c_cp)),
-                ("pool_full", c_i64), ("launches", c_i64)]
+                ("pool_full", c_i64), ("launches", c_i64), ("raw_staged", c_i64)]
 
 
 class PeriodStats(ctypes.Structure):

@@ -63,6 +63,7 @@ class EnsembleResult:
     cuts_final: int = -1    # cuts [0, cuts_final) are final (T after finalize; a snapshot may be less)
     pool_full: int = 0      # overflowed instances frozen by a full compartment pool (R20)
     launches: int = 1       # kernels the simulation launched (SSA + compaction)
+    raw_staged: int = 0     # raw cuts staged per lane in shared memory (option raw_stage)
 
     @property
     def frozen_fraction(self) -> float:
@@ -301,6 +302,7 @@ class Model:
             reactions=st.reactions, absorbed=st.absorbed, overflowed=st.overflowed, finished=st.finished,
             kernel_ms=st.kernel_ms, species=[st.species_names[s].decode() for s in range(S)],
             cuts_final=st.cuts_final, pool_full=st.pool_full, launches=st.launches,
+            raw_staged=st.raw_staged,
         )
 
     def snapshot(self):

@@ -257,6 +257,9 @@ cwc_status cwc_set_option_i64(cwc_model_t m, const char* key, int64_t v) {
         } else if (k == "smem_stats") {
             need(v >= 0 && v <= 3, "smem_stats is 0 (global), 1 (auto), 2 (sparse) or 3 (dense)");
             m->smem_stats = (int)v;
+        } else if (k == "raw_stage") {
+            need(v == 0 || v == 1, "raw_stage is 0 or 1");
+            m->raw_stage = (int)v;
         } else if (k == "ilp") {
             need(v == 1 || v == 2, "ilp is 1 or 2");
             m->ilp = (int)v;
@@ -462,6 +465,7 @@ cwc_status cwc_stats(cwc_model_t m, cwc_stats_t* out) {
         out->finished = ctr[CWC_CTR_FINISHED];
         out->pool_full = ctr[CWC_CTR_POOL_FULL];
         out->launches = m->launches;
+        out->raw_staged = m->raw_stage_now;
         out->kernel_ms = m->kernel_ms;
         out->cuts_final = m->cuts_final;
         out->species_names = m->name_ptrs.data();

@@ -42,6 +42,11 @@ struct cwc_params {
     // item count is *n_items_dev (written by the previous launch's compaction), else n_items
     const unsigned int* list;
     const unsigned long long* n_items_dev;
+    // raw-cut staging (1 = on): each lane collects the 8 cuts of one 32-byte block of the
+    // time-blocked raw layout in dynamic shared memory (at byte raw_stage_off: [blockDim][S][8]
+    // int32, then one u32 slot mask per lane) and writes the block as whole 32-byte sectors
+    int raw_stage;
+    int raw_stage_off;
 };
 
 #define CWC_TERMINAL 0x80000000u

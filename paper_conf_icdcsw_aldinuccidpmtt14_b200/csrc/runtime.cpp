@@ -27,7 +27,7 @@
 #endif
 
 // bench.py counts the launch parameter block in its end-to-end H2D bytes (PARAM_BYTES)
-static_assert(sizeof(cwc_params) == 272, "cwc_params layout changed: update bench.py PARAM_BYTES");
+static_assert(sizeof(cwc_params) == 280, "cwc_params layout changed: update bench.py PARAM_BYTES");
 static_assert(sizeof(cwc_logtab_entry) * 128 == 3072, "log table size");
 
 namespace {
@@ -539,6 +539,18 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
         ckd(d.FuncSetAttribute(m->function, CU_FUNC_ATTRIBUTE_MAX_DYNAMIC_SHARED_SIZE_BYTES, (int)dyn_smem),
             "dynamic smem");
     }
+    // raw-cut staging: a lane's 8 cuts of one time block go to DRAM as whole 32-byte sectors
+    // instead of eight 4-byte stores that L2 may write back (and re-read for ECC fill) before the
+    // sector is complete (LV 1M: 8.3 GB of DRAM traffic per launch for 4.0 GB of raw cuts)
+    int raw_stage = 0, raw_stage_off = 0;
+    if (need_raw && m->raw_stage && m->ilp == 1) {
+        const size_t off = (dyn_smem + 15) / 16 * 16;
+        const size_t bytes = off + (size_t)m->block_threads * ((size_t)S * CWC_RAW_BLOCK * 4 + 4);
+        if (fits(bytes)) raw_stage = 1, raw_stage_off = (int)off, dyn_smem = bytes;
+        ckd(d.FuncSetAttribute(m->function, CU_FUNC_ATTRIBUTE_MAX_DYNAMIC_SHARED_SIZE_BYTES, (int)dyn_smem),
+            "dynamic smem");
+    }
+    m->raw_stage_now = raw_stage;
     int per_sm = m->blocks_per_sm > 0 ? std::min(m->blocks_per_sm, occ) : occ;
     int64_t grid = (int64_t)sms * per_sm;
     // Every resident slot is launched even when there are fewer instances than lanes: warps race
@@ -612,6 +624,8 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     m->cancel_requested = false;
     P.logtab = m->d_logtab;
     P.smem_stats = smem_mode;
+    P.raw_stage = raw_stage;
+    P.raw_stage_off = raw_stage_off;
 
     if (!resume) {
         ck(cudaMemsetAsync(m->d_stats, 0, need_stats * 8, stream), "memset(stats)");

@@ -32,6 +32,8 @@ struct cwc_model {
     int ilp = 1;
     int delta_table = -1;
     int smem_stats = 1;
+    int raw_stage = 1;                    // raw-cut staging in shared memory (1 = when it fits)
+    int raw_stage_now = 0;                // whether the last launch staged
     // cut recording inside the fast step (1) or on the full-step path (0); -1 = auto: by the
     // reactions per recorded cut of the last simulation on this handle (else a0(x0) * dt)
     int fast_cut = -1;

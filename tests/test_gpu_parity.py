@@ -240,6 +240,27 @@ def test_statistics_staging_invariance(name, n):
                 assert np.array_equal(a, b), mode
 
 
+@pytest.mark.parametrize("opts", [{}, {"quantum_samples": 5}, {"quantum_samples": 13, "block_threads": 256},
+                                  {"refill": False, "quantum_samples": 3}, {"compact": 1}, {"fast_cut": 1}])
+def test_raw_staging_invariance(opts):
+    """Raw cuts staged per lane in shared memory and written as whole 32-byte blocks (option
+    raw_stage, the default) equal the direct 4-byte stores and the oracle: blocks cut by quanta
+    that are not multiples of 8 cuts, absorbed instances (cuts to K in one go), overflowed ones
+    (the staged part of a block, then -1) and a ragged last block (T = 101)."""
+    cfg = W.CONFIGS["lv"]
+    n, t_end, dt, seed = 600, 50.0, 0.5, cfg.seed + 7
+    on, raw_on, fl_on, re_on, _ = gpu_run(cfg.model, n, 0, n, t_end, dt, seed, hist_bins=cfg.hist_bins,
+                                          hist_width=cfg.hist_width, **opts)
+    off, raw_off, fl_off, re_off, _ = gpu_run(cfg.model, n, 0, n, t_end, dt, seed, hist_bins=cfg.hist_bins,
+                                              hist_width=cfg.hist_width, raw_stage=0, **opts)
+    assert on.raw_staged == 1 and off.raw_staged == 0
+    assert on.absorbed > 0 and on.overflowed > 0
+    assert np.array_equal(raw_on, raw_off) and np.array_equal(fl_on, fl_off) and np.array_equal(re_on, re_off)
+    orun = _oracle(cfg.model, 0, n, t_end, dt, seed)
+    assert np.array_equal(raw_on, orun.raw)
+    assert_matches_oracle_stats(on, orun.raw, QS)
+
+
 def test_sparse_ticket_overflow_goes_global(monkeypatch):
     """Sparse staging admits at most CWC_SPARSE_TICKETS work items of one quantum per CTA to its
     16-bit limbs; later items record to global memory.  With the limit lowered to 64 most records
