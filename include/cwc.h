@@ -166,6 +166,10 @@ cwc_status cwc_model_info(cwc_model_t m, cwc_model_info_t* out);
  *                        dense per-CTA shared moments (u64, T*(1+3S)*8 bytes); 1 auto = sparse,
  *                        else dense, else global — each only when it fits without lowering
  *                        residency.  Results are bit-identical.                  default 1
+ *   "draw_batch"         -1/0/2..8: draws per inner-loop trip — the Philox blocks and CWC-logs of
+ *                        the next D steps as D independent chains, then D fast steps (0: the
+ *                        next draw inside each fast step); -1 = auto: 4 up to 8 species, 3 up to
+ *                        16, else 0.  Performance only: results are bit-identical.   default -1
  *   "raw_stage"          0/1: a lane collects the 8 cuts of one 32-byte block of the raw layout in
  *                        shared memory and writes the block as whole sectors (1: when it fits
  *                        without lowering residency and ilp = 1).  Results are bit-identical.

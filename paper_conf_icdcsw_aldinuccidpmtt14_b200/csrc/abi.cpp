@@ -257,6 +257,9 @@ cwc_status cwc_set_option_i64(cwc_model_t m, const char* key, int64_t v) {
         } else if (k == "smem_stats") {
             need(v >= 0 && v <= 3, "smem_stats is 0 (global), 1 (auto), 2 (sparse) or 3 (dense)");
             m->smem_stats = (int)v;
+        } else if (k == "draw_batch") {
+            need(v == -1 || v == 0 || (v >= 2 && v <= 8), "draw_batch is -1 (auto), 0 or 2..8");
+            m->draw_batch = (int)v;
         } else if (k == "raw_stage") {
             need(v == 0 || v == 1, "raw_stage is 0 or 1");
             m->raw_stage = (int)v;

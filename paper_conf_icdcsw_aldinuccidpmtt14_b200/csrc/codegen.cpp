@@ -30,12 +30,21 @@ std::string generate_model_section(const FlatModel& fm, const KernelConfig& cfg)
       << "\n#define CWC_BLOCK " << cfg.block_threads << "\n#define CWC_MINB " << cfg.min_blocks << "\n#define CWC_ILP " << cfg.ilp << "\n";
     o << "#define CWC_PERIOD_S " << cfg.period_species << "\n#define CWC_PERIOD_LO " << cfg.period_lo
       << "LL\n#define CWC_PERIOD_HI " << cfg.period_hi << "LL\n";
+    o << "#define CWC_RAW " << (cfg.raw ? 1 : 0) << "  // raw cuts recorded (option raw_samples)\n";
     o << "#define CWC_X_CAP " << cfg.x_cap << "\n#define CWC_FAST_CUT " << (cfg.fast_cut ? 1 : 0) << "\n";
     o << "#define CWC_SENTINEL " << fm.sentinel << "  // species \"#full\" of the compartment pools (R20), -1 none\n";
     // branch-free fast commit (cuts on the full-step path) for small models: the select per state
     // word costs less than the divergent branch up to ~4 species (same-box A/B, profiles/
     // r2_ab_kernel.log: LV 1M +2.7 %, 100k +3.3 %; circadian, 9 species, -4 %)
-    o << "#ifndef CWC_BRANCHFREE\n#define CWC_BRANCHFREE " << (S <= 4 ? 1 : 0) << "\n#endif\n\n";
+    o << "#ifndef CWC_BRANCHFREE\n#define CWC_BRANCHFREE " << (S <= 4 ? 1 : 0) << "\n#endif\n";
+    // draw batch: the next D draws as D independent chains, then D fast steps (same-box sweep,
+    // profiles/s2f_ab_draw_batch.log: D = 4 best up to 8 species (LV +3.5-4.1 %, Neurospora +6 %,
+    // Schlogl +1 %), 3 for 9-16 (compartments +5.3 %, circadian +7.3 %); larger models keep 0)
+    const int db = cfg.draw_batch >= 0 ? cfg.draw_batch : (S <= 8 ? 4 : (S <= 16 ? 3 : 0));
+    o << "#ifndef CWC_DRAW_BATCH\n#define CWC_DRAW_BATCH " << (cfg.ilp == 1 ? db : 0) << "\n#endif\n";
+    // the batch's draws are committed to the lane state when the warp leaves the loop (LV 1M +6 %,
+    // circadian +1.5 %, Neurospora +1 %) — except for one-species models (Schlogl -2.7 %), same box
+    o << "#ifndef CWC_DEFER_DRAW\n#define CWC_DEFER_DRAW " << (S > 1 ? 1 : 0) << "\n#endif\n\n";
     if (cfg.seed_keys) {
         const uint32_t k0 = (uint32_t)cfg.seed, k1 = (uint32_t)(cfg.seed >> 32);
         o << "#define CWC_STATIC_KEYS 1\nstatic constexpr cwc_round_keys cwc_rk_static = {{";

@@ -20,6 +20,8 @@ struct KernelConfig {
     int64_t period_lo = 0, period_hi = 1;
     int64_t x_cap = 0;
     bool fast_cut = true;  // the fast step records a due cut itself (else it leaves the fast loop)
+    bool raw = true;       // raw cuts may be recorded (else every raw-cut path is compiled out)
+    int draw_batch = -1;   // draws per inner-loop trip (0 = one per fast step; -1 = auto by species)
     std::vector<int64_t> hist_lo, hist_width;  // [S]
 };
 

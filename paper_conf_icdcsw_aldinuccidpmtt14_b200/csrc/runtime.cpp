@@ -275,6 +275,8 @@ void compile(cwc_model* m, const uint64_t* seed) {
     cfg.hist_bins = m->hist_bins;
     cfg.x_cap = m->x_cap;
     cfg.fast_cut = m->fast_cut >= 0 ? m->fast_cut != 0 : m->fast_cut_now;  // explicit option wins
+    cfg.draw_batch = m->draw_batch;
+    cfg.raw = m->raw_samples != 0;
     cfg.hist_lo = m->hist_lo;
     cfg.hist_width = m->hist_width;
     if (seed && m->seed_jit) {
@@ -1085,6 +1087,7 @@ void selftest_step(cwc_model* m, int64_t n, int32_t n_draws, const int32_t* x, c
     for (int64_t i = 0; i < n; ++i)
         if (k[i] < 0 || k[i] > T) fail(CWC_E_INVALID, "next cut index outside [0, K+1]");
     if (n == 0) return;
+    if (!m->raw_samples) fail(CWC_E_STATE, "the self-test records cuts: raw_samples must be on");
     compile(m, nullptr);
     const int dev = current_device(m);
     ensure_module(m, dev);

@@ -32,6 +32,7 @@ struct cwc_model {
     int ilp = 1;
     int delta_table = -1;
     int smem_stats = 1;
+    int draw_batch = -1;                  // draws per inner-loop trip (0, 2..8; -1 auto)
     int raw_stage = 1;                    // raw-cut staging in shared memory (1 = when it fits)
     int raw_stage_now = 0;                // whether the last launch staged
     // cut recording inside the fast step (1) or on the full-step path (0); -1 = auto: by the

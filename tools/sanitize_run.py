@@ -31,6 +31,11 @@ def main():
         (W.COMPARTMENTS, 200, 2.0, 0.5, {"smem_stats": 3}),
         (W.LOTKA_VOLTERRA, 300, 0.3, 0.05, {"compact": 1, "quantum_samples": 2}),
         (W.SCHLOGL, 500, 0.5, 0.05, {"refill": False, "quantum_samples": 3}),
+        # round 2, second half: raw-cut staging with blocks cut by quanta (partial flushes), the
+        # draw-batch loop (default) against the per-step draw, no staging
+        (W.LOTKA_VOLTERRA, 300, 0.3, 0.05, {"quantum_samples": 3}),
+        (W.LOTKA_VOLTERRA, 300, 0.3, 0.05, {"draw_batch": 0, "raw_stage": 0}),
+        (W.CIRCADIAN, 200, 4.0, 0.5, {"draw_batch": 2}),
     ]
     for md, n, t_end, dt, opts in runs:
         m = cwc.Model.from_def(md, hist_bins=64, **opts)
