@@ -261,6 +261,20 @@ def test_raw_staging_invariance(opts):
     assert_matches_oracle_stats(on, orun.raw, QS)
 
 
+def test_bounds_checked_kernel():
+    """Every shared-memory and global index of the SSA kernel bounds-checked on the device
+    (CWC_CHECKS=1, a violation traps) over raw-cut staging with partial blocks, the three
+    statistics layouts, lockstep / compacted launches, pools and a 20,001-cut horizon; results
+    equal the oracle's.  Own process: a trap poisons the CUDA context."""
+    import os
+    import subprocess
+    import sys
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    r = subprocess.run([sys.executable, os.path.join(root, "tests", "workers", "bounds_check.py")],
+                       capture_output=True, text=True, timeout=900)
+    assert r.returncode == 0 and "BOUNDS OK" in r.stdout, r.stdout[-2000:] + r.stderr[-2000:]
+
+
 def test_sparse_ticket_overflow_goes_global(monkeypatch):
     """Sparse staging admits at most CWC_SPARSE_TICKETS work items of one quantum per CTA to its
     16-bit limbs; later items record to global memory.  With the limit lowered to 64 most records
