@@ -44,7 +44,13 @@ std::string generate_model_section(const FlatModel& fm, const KernelConfig& cfg)
     o << "#ifndef CWC_DRAW_BATCH\n#define CWC_DRAW_BATCH " << (cfg.ilp == 1 ? db : 0) << "\n#endif\n";
     // the batch's draws are committed to the lane state when the warp leaves the loop (LV 1M +6 %,
     // circadian +1.5 %, Neurospora +1 %) — except for one-species models (Schlogl -2.7 %), same box
-    o << "#ifndef CWC_DEFER_DRAW\n#define CWC_DEFER_DRAW " << (S > 1 ? 1 : 0) << "\n#endif\n\n";
+    o << "#ifndef CWC_DEFER_DRAW\n#define CWC_DEFER_DRAW " << (S > 1 ? 1 : 0) << "\n#endif\n";
+    // cooperative cut recording in the fast step (same-box A/B, profiles/s2p_ab_coop_emission.log):
+    // it pays when a cut is recorded by few lanes of a warp at a time and its species spread over
+    // the lanes — compartments (9 species, a cut every ~290 reactions) +4.4 % — and loses where
+    // many lanes record at once (vesicles, 29 species: -40 %) or the cut has 1-3 species
+    // (Schlogl, Neurospora: -7 %)
+    o << "#ifndef CWC_COOP_EMIT\n#define CWC_COOP_EMIT " << (S >= 8 && S <= 16 ? 1 : 0) << "\n#endif\n\n";
     if (cfg.seed_keys) {
         const uint32_t k0 = (uint32_t)cfg.seed, k1 = (uint32_t)(cfg.seed >> 32);
         o << "#define CWC_STATIC_KEYS 1\nstatic constexpr cwc_round_keys cwc_rk_static = {{";
@@ -277,6 +283,16 @@ std::string generate_model_section(const FlatModel& fm, const KernelConfig& cfg)
     o << "        default: break;\n    }\n";
     o << "    const long long d = (long long)v - lo;\n";
     o << "    if (d < 0) return 0;\n    const long long b = d / w;\n    return b >= CWC_B ? CWC_B + 1 : (int)b + 1;\n}\n";
+    // the same bins with a run-time species index (cooperative cut recording: lane s records
+    // species s), from a shared-memory copy of (lo, width)
+    o << "__constant__ long long cwc_hist_c[" << 2 * S << "] = {";
+    for (int s = 0; s < S; ++s) o << (s ? ", " : "") << cfg.hist_lo[s] << "LL, " << cfg.hist_width[s] << "LL";
+    o << "};\n__shared__ long long cwc_hist_sm[" << 2 * S << "];\n";
+    o << "__device__ __forceinline__ void cwc_hist_init() {\n    for (int i = threadIdx.x; i < " << 2 * S
+      << "; i += blockDim.x) cwc_hist_sm[i] = cwc_hist_c[i];\n}\n";
+    o << "__device__ __forceinline__ int cwc_bin_rt(int s, int v) {\n"
+         "    const long long d = (long long)v - cwc_hist_sm[2 * s];\n    if (d < 0) return 0;\n"
+         "    const long long b = d / cwc_hist_sm[2 * s + 1];\n    return b >= CWC_B ? CWC_B + 1 : (int)b + 1;\n}\n";
     o << "// ---- end of generated model section\n\n";
     return o.str();
 }

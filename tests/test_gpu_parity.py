@@ -275,6 +275,23 @@ def test_bounds_checked_kernel():
     assert r.returncode == 0 and "BOUNDS OK" in r.stdout, r.stdout[-2000:] + r.stderr[-2000:]
 
 
+@pytest.mark.parametrize("name,defines", [("compartments", ""), ("compartments", "CWC_SPARSE_TICKETS=64"),
+                                           ("vesicles", "CWC_COOP_EMIT=1"),
+                                           ("vesicles", "CWC_COOP_EMIT=1;CWC_SPARSE_TICKETS=64")])
+def test_cooperative_cut_recording(monkeypatch, name, defines):
+    """Cuts recorded cooperatively by the warp in the fast step (raw cuts off, sparse statistics:
+    lane s records species s of each due lane's cut; compartments by default, vesicles forced),
+    including records beyond the sparse admission limit (global path): statistics equal the
+    oracle's statistics of its own samples."""
+    cfg = W.CONFIGS[name]
+    n, t_end = 6000, 30.0
+    if defines:
+        monkeypatch.setenv("CWC_KERNEL_DEFINES", defines)
+    res, *_ = gpu_run(cfg.model, n, 0, n, t_end, cfg.sample_dt, cfg.seed, hist_bins=cfg.hist_bins,
+                      hist_width=cfg.hist_width, raw=False, fast_cut=1, quantum_samples=16)
+    assert_matches_oracle_stats(res, _oracle(cfg.model, 0, n, t_end, cfg.sample_dt, cfg.seed).raw, QS)
+
+
 def test_sparse_ticket_overflow_goes_global(monkeypatch):
     """Sparse staging admits at most CWC_SPARSE_TICKETS work items of one quantum per CTA to its
     16-bit limbs; later items record to global memory.  With the limit lowered to 64 most records
