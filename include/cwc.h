@@ -154,7 +154,10 @@ cwc_status cwc_model_info(cwc_model_t m, cwc_model_info_t* out);
  *                        whole trajectories up to one instance per resident lane, else 32
  *                        (up to 4 per lane) or 8 quanta, rounded up to a multiple of 8 cuts.
  *                        Scheduling only: results are bit-identical for every value (R12).
- *   "block_threads"      CUDA block size (multiple of 32, <= 1024).              default 768
+ *   "block_threads"      CUDA block size (multiple of 32, <= 1024).  Default: auto per launch —
+ *                        768 (80 registers) from 1.5 instances per resident lane up, else 512
+ *                        (113 registers; the instances then exceed the lanes and quanta balance
+ *                        the load).
  *   "blocks_per_sm"      persistent CTAs per SM; 0 = occupancy maximum.          default 0
  *   "min_blocks"         register budget: __launch_bounds__ min CTAs per SM; 0 = auto
  *                        (768 / block_threads, i.e. <= 80 registers).

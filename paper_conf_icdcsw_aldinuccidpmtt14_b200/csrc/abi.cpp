@@ -231,6 +231,7 @@ cwc_status cwc_set_option_i64(cwc_model_t m, const char* key, int64_t v) {
         } else if (k == "block_threads") {
             need(v >= 32 && v <= 1024 && v % 32 == 0, "block_threads: multiple of 32 in [32, 1024]");
             m->block_threads = (int)v;
+            m->block_auto = false;
         } else if (k == "period_species") {
             need(v >= -1 && v < m->fm.S(), "period_species: flat species index or -1");
             m->period_species = (int)v;

@@ -475,6 +475,18 @@ void simulate_range(cwc_model* m, int64_t n_total, int64_t first, int64_t count,
     const int64_t T = K + 1;
     const int S = m->fm.S();
     m->fast_cut_now = choose_fast_cut(m, dt);
+    // auto CTA size (same-box sweep, profiles/s2r_ab_block_sizes.log, s2s_ab_block_underfilled.log):
+    // 768 threads x 80 registers when the instances fill the lanes at least 1.5 times over; below,
+    // 512 x 113 registers — the instances then exceed the fewer lanes, so simulation quanta balance
+    // the load, and each warp runs a better-scheduled step (LV 100k 969 -> 838 ms, 125k 1065 ->
+    // 1034 ms; at 250k-1M and on the 1M configs 768 is best or equal)
+    if (m->block_auto && m->ilp == 1) {
+        int dv = m->device, sms = 0;
+        if (dv < 0 && cudaGetDevice(&dv) != cudaSuccess) dv = -1;
+        if (dv >= 0 && cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dv) != cudaSuccess) sms = 0;
+        cudaGetLastError();
+        if (sms > 0) m->block_threads = count * 2 < (int64_t)sms * 768 * 3 ? 512 : 768;
+    }
     compile(m, &seed);
     const int dev = current_device(m);
     ensure_module(m, dev);

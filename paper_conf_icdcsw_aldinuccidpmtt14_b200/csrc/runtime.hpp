@@ -27,6 +27,7 @@ struct cwc_model {
     int seed_jit = 0;
     std::vector<int64_t> hist_lo, hist_width;
     int64_t quantum_samples = 0;
+    bool block_auto = true;               // CTA size chosen per launch (until block_threads is set)
     int block_threads = 768;  // one 24-warp CTA per SM (measured best: LV 1.13 vs 1.21 s at 3 x 256)
     int min_blocks = 0;
     int ilp = 1;
